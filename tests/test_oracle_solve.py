@@ -1,0 +1,173 @@
+"""Pins for the oracle's CG / CPPCG solves (CPU, no GPU).
+
+The method reaches u* = A^{-1} u^n (A is SPD, so the solution is unique); CG and
+CPPCG are two routes to it. Pins:
+
+* dense direct solve (numpy LAPACK) on <= 16x16 meshes, several dt (conditioning);
+* DCT-II diagonalisation for uniform density at any size (closed form);
+* nx = 1: tridiagonal (Thomas / LAPACK banded) solve;
+* invariants: sum(u) conserved at EVERY iteration under reflective boundaries
+  (1^T r_0 = 0, A 1 = 1); discrete maximum principle (A is an M-matrix with unit
+  row sums); monotone A-norm error of CG (CG minimises it over the Krylov space);
+* eq (6) iteration bound, with kappa from the dense spectrum;
+* CPPCG field == CG field (same system).
+"""
+import numpy as np
+import pytest
+import scipy.fft
+import scipy.linalg
+
+from paper_conf_cluster_mcintosh_smithm17_b200 import inputs
+from test_oracle_operator import dense_A, deck_coeffs
+
+
+def setup(ora, d):
+    Kx, Ky = deck_coeffs(ora, d)
+    u0 = d.density * d.energy
+    return Kx, Ky, u0
+
+
+SMALL = [("pipe", 16, 16, 0, 0.004), ("random", 16, 16, 1, 0.4), ("random", 13, 11, 2, 4.0),
+         ("random", 12, 12, 3, 40.0), ("random", 16, 5, 4, 4.0)]
+
+
+@pytest.mark.parametrize("kind,nx,ny,seed,dt", SMALL)
+@pytest.mark.parametrize("method", [0, 1])
+def test_dense_direct_solve(ora, kind, nx, ny, seed, dt, method):
+    d = (inputs.random_fields(nx, ny, seed, dt=dt) if kind == "random"
+         else inputs.crooked_pipe(nx, ny))
+    Kx, Ky, u0 = setup(ora, d)
+    A = dense_A(ora, Kx, Ky, nx, ny)
+    ustar = np.linalg.solve(A, u0.ravel()).reshape(ny, nx)
+    res = ora.solve(Kx, Ky, u0, method=method, eps=1e-15, max_iters=5000, inner_steps=4,
+                    presteps=8)
+    assert res.status == 0
+    err = np.abs(res.u - ustar).max() / np.abs(ustar).max()
+    assert err <= 1e-11, err
+
+
+@pytest.mark.parametrize("nx,ny,rho,method", [(96, 64, 1.0, 0), (64, 96, 0.1, 1),
+                                              (80, 80, 2.0, 1)])
+def test_uniform_density_dct_solve(ora, nx, ny, rho, method):
+    d = inputs.uniform_fields(nx, ny, rho=rho, seed=7)
+    rx, ry = ora.mesh_r(d)
+    Kx, Ky, u0 = setup(ora, d)
+    i, j = np.arange(nx), np.arange(ny)
+    lam = (1.0 + 4 * (rx / rho) * np.sin(np.pi * i / (2 * nx))[None, :] ** 2
+           + 4 * (ry / rho) * np.sin(np.pi * j / (2 * ny))[:, None] ** 2)
+    ustar = scipy.fft.idctn(scipy.fft.dctn(u0, type=2, norm="ortho") / lam, type=2,
+                            norm="ortho")
+    res = ora.solve(Kx, Ky, u0, method=method, eps=1e-14, max_iters=20000, inner_steps=6)
+    assert res.status == 0
+    assert np.abs(res.u - ustar).max() / np.abs(ustar).max() <= 1e-11
+
+
+@pytest.mark.parametrize("method", [0, 1])
+def test_single_column_thomas(ora, method):
+    d = inputs.random_fields(1, 200, seed=11, dt=0.4)
+    Kx, Ky, u0 = setup(ora, d)
+    ky = Ky[:, 0]  # faces 0..ny
+    diag = 1.0 + ky[1:] + ky[:-1]
+    ab = np.zeros((3, 200))
+    ab[0, 1:] = -ky[1:-1]
+    ab[1] = diag
+    ab[2, :-1] = -ky[1:-1]
+    ustar = scipy.linalg.solve_banded((1, 1), ab, u0[:, 0])
+    res = ora.solve(Kx, Ky, u0, method=method, eps=1e-15, max_iters=5000, inner_steps=3,
+                    presteps=10)
+    assert res.status == 0
+    np.testing.assert_allclose(res.u[:, 0], ustar, rtol=1e-10)
+
+
+@pytest.mark.parametrize("method,ks", [(0, range(1, 40, 3)), (1, [31, 32, 35, 40, 45])])
+def test_conservation_every_iteration(ora, method, ks):
+    d = inputs.crooked_pipe(32)
+    Kx, Ky, u0 = setup(ora, d)
+    s0 = u0.sum()
+    for k in ks:
+        res = ora.solve(Kx, Ky, u0, method=method, eps=0.0, max_iters=k, inner_steps=5)
+        assert res.stats["iterations"] == k
+        assert abs(res.u.sum() - s0) / s0 <= 1e-13
+
+
+@pytest.mark.parametrize("kind,seed", [("pipe", 0), ("random", 3)])
+def test_maximum_principle(ora, kind, seed):
+    d = inputs.crooked_pipe(48) if kind == "pipe" else inputs.random_fields(40, 30, seed)
+    Kx, Ky, u0 = setup(ora, d)
+    for method in (0, 1):
+        res = ora.solve(Kx, Ky, u0, method=method, eps=1e-14, max_iters=20000)
+        tol = 1e-10 * np.abs(u0).max()
+        assert res.u.min() >= u0.min() - tol
+        assert res.u.max() <= u0.max() + tol
+
+
+@pytest.mark.parametrize("nx,dt", [(16, 4.0), (16, 0.4), (12, 40.0)])
+def test_cg_monotone_A_norm_error(ora, nx, dt):
+    """Reading R16: ||r|| is not monotone in CG, the A-norm error is."""
+    d = inputs.random_fields(nx, nx, seed=2, dt=dt)
+    Kx, Ky, u0 = setup(ora, d)
+    A = dense_A(ora, Kx, Ky, nx, nx)
+    ustar = np.linalg.solve(A, u0.ravel())
+    e0 = u0.ravel() - ustar
+    E0 = np.sqrt(e0 @ A @ e0)
+    prev = E0
+    for k in range(1, 400):
+        res = ora.solve(Kx, Ky, u0, method=0, eps=0.0, max_iters=k)
+        e = res.u.ravel() - ustar
+        E = np.sqrt(max(e @ A @ e, 0.0))
+        if prev < 1e-10 * E0:
+            break
+        assert E <= prev * (1 + 1e-12), (k, E, prev)
+        prev = E
+
+
+@pytest.mark.parametrize("n", [16, 24])
+def test_cg_iteration_bound_eq6(ora, n):
+    """eq (6): k <= sqrt(kappa)/2 ln(2/eps_A); for a residual test ||r_k|| < eps ||r_0||
+    the A-norm reduction needed is eps/sqrt(kappa)."""
+    d = inputs.crooked_pipe(n)
+    Kx, Ky, u0 = setup(ora, d)
+    ev = np.linalg.eigvalsh(dense_A(ora, Kx, Ky, n, n))
+    kappa = ev[-1] / ev[0]
+    for eps in (1e-6, 1e-10, 1e-13):
+        res = ora.solve(Kx, Ky, u0, method=0, eps=eps, max_iters=100000)
+        bound = np.sqrt(kappa) / 2 * np.log(2 * np.sqrt(kappa) / eps)
+        assert res.stats["iterations"] <= np.ceil(bound)
+
+
+@pytest.mark.parametrize("n,s", [(64, 10), (64, 3), (48, 1), (40, 6)])
+def test_cppcg_equals_cg(ora, n, s):
+    d = inputs.crooked_pipe(n)
+    Kx, Ky, u0 = setup(ora, d)
+    cg = ora.solve(Kx, Ky, u0, method=0, eps=1e-15, max_iters=100000)
+    pp = ora.solve(Kx, Ky, u0, method=1, eps=1e-15, max_iters=100000, inner_steps=s)
+    assert cg.status == 0 and pp.status == 0
+    assert pp.stats["presteps"] == 30 and pp.stats["outer"] > 0
+    assert np.abs(pp.u - cg.u).max() / np.abs(cg.u).max() <= 1e-12
+    # communication avoidance: far fewer outer iterations (dot products)
+    assert pp.stats["outer"] * (s + 1) >= 0.5 * (cg.stats["iterations"] - 30)
+    if s >= 3:
+        assert pp.stats["outer"] < cg.stats["iterations"] - 30
+
+
+def test_zero_residual_returns_immediately(ora):
+    d = inputs.uniform_fields(8, 8, rho=1.0, dt=0.0)  # dt = 0 -> A = I exactly
+    Kx, Ky, u0 = setup(ora, d)
+    for m in (0, 1):
+        res = ora.solve(Kx, Ky, u0, method=m, eps=1e-10, max_iters=10)
+        assert res.status == 0 and res.stats["iterations"] == 0
+        assert np.array_equal(res.u, u0)
+
+
+def test_not_converged_and_bad_args(ora):
+    d = inputs.crooked_pipe(32)
+    Kx, Ky, u0 = setup(ora, d)
+    res = ora.solve(Kx, Ky, u0, method=0, eps=1e-15, max_iters=5)
+    assert res.status == 1 and res.stats["iterations"] == 5
+    res = ora.solve(Kx, Ky, u0, method=1, eps=1e-15, max_iters=12, presteps=30)
+    assert res.status == 1 and res.stats["iterations"] == 12 and res.stats["outer"] == 0
+    d = inputs.crooked_pipe(128)
+    Kx, Ky, u0 = setup(ora, d)
+    res = ora.solve(Kx, Ky, u0, method=1, eps=1e-15, max_iters=32, presteps=30)
+    assert res.status == 1 and res.stats["outer"] == 2
+    assert ora.solve(Kx, Ky, u0, method=1, inner_steps=0).status == -1
