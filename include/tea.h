@@ -1,0 +1,181 @@
+/*
+ * tea.h -- C ABI of the B200-native TeaLeaf CG / CPPCG hot path.
+ *
+ * One implicit timestep of 2D heat conduction (Sec. II):
+ * solve (I + dt L) u^{n+1} = u^n with the matrix-free 5-point operator of
+ * Listing 1 (L349-367), by CG (Sec. III.A) or by Chebyshev
+ * polynomially preconditioned CG, CPPCG (Sec. III.B-D), on a mesh that
+ * may be split into px x py rectangular blocks (Sec. IV.A) exchanging
+ * halos of depth d (matrix powers, Sec. IV.C.2).
+ *
+ * All compute runs in hand-written sm_100a CUDA kernels inside this library.
+ * Caller memory in the signatures is plain pointers: HOST pointers for the
+ * global input/output fields, a DEVICE pointer for the workspace (the caller,
+ * e.g. PyTorch, owns it; the library never frees it).
+ *
+ * Global field layout (density, energy, u_host): nx*ny doubles, row-major,
+ * x fastest: cell (j,k) at index k*nx + j, j in [0,nx), k in [0,ny).
+ *
+ * Errors: every call returns a tea_status. Negative = failure; the context is
+ * then unusable except for tea_last_error() and tea_finalize(). A positive
+ * TEA_NOT_CONVERGED means max_iters was reached; the fields are valid.
+ * Not thread-safe per context. All calls on one context must come from one host
+ * thread; different contexts are independent.
+ */
+#ifndef TEA_H
+#define TEA_H
+
+#include <stddef.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+#define TEA_ABI_VERSION 1
+
+typedef enum {
+    TEA_OK = 0,
+    TEA_NOT_CONVERGED = 1,
+    TEA_ERR_ARG = -1,       /* bad argument: sizes, decomposition, depth, workspace   */
+    TEA_ERR_CUDA = -2,      /* CUDA runtime error (message in tea_last_error)          */
+    TEA_ERR_NCCL = -3,      /* NCCL error                                              */
+    TEA_ERR_BREAKDOWN = -4, /* p.w <= 0, non-finite scalar, or bad eigen-estimate      */
+    TEA_ERR_STATE = -5      /* call out of order / context already failed             */
+} tea_status;
+
+typedef enum { TEA_CG = 0, TEA_CPPCG = 1 } tea_method;
+
+typedef struct tea_ctx tea_ctx; /* opaque, library-owned */
+
+/* Mesh: nx x ny cells on [xmin,xmax] x [ymin,ymax]; dx = (xmax-xmin)/nx,
+ * dy = (ymax-ymin)/ny; rx = dt/dx^2, ry = dt/dy^2 (BASELINE.json north_star). */
+typedef struct {
+    int nx, ny;
+    double xmin, xmax, ymin, ymax;
+} tea_mesh;
+
+/* Decomposition: px x py blocks, block b = by*px + bx owns the
+ * columns/rows given by an even split with the remainder on low-index blocks.
+ * The blocks are shared evenly by `nranks` processes (one process per GPU):
+ * rank r owns blocks [r*B, (r+1)*B), B = px*py/nranks. nranks == 1 with
+ * px*py > 1 runs every block in this process on one GPU (halo transport by
+ * device copies instead of NCCL -- same pack/unpack kernels).
+ * halo_depth d >= 1: matrix-powers depth of the CPPCG inner loop.
+ * nccl_id: 128-byte ncclUniqueId from tea_get_nccl_id() on rank 0, broadcast by
+ * the caller; NULL when nranks == 1. Pass NULL for `dist` to get 1x1, d = 1.  */
+typedef struct {
+    int rank, nranks;
+    int px, py;
+    int halo_depth;
+    const void *nccl_id;
+} tea_dist;
+
+/* Solver options (DESIGN.md readings). Pass NULL for the defaults in brackets. */
+typedef struct {
+    int presteps;           /* CG iterations before CPPCG switches (R6)        [30]   */
+    double eig_margin_lo;   /* lambda_min = lo * min Ritz value (R8)           [0.95] */
+    double eig_margin_hi;   /* lambda_max = hi * max Ritz value (R8)           [1.05] */
+    int mean_mode;          /* face coefficient: 0 rx*mean(1/rho) (R1), 1 rx*mean(rho) [0] */
+    int loop_mode;          /* 0 device WHILE graph, 1 chunked graphs, 2 eager  [0]    */
+    int check_interval;     /* iterations per chunk in loop_mode 1/2 (0 = auto) [0]    */
+    int profile;            /* 1: eager launches timed per kernel (tea_kernel_times)[0]*/
+    int tile_rows;          /* rows per CTA tile of the stencil kernels, 0 = auto [0]  */
+} tea_opts;
+
+/* Per-solve statistics. */
+typedef struct {
+    int iterations;    /* CG iterations (CG) or presteps + outer iterations (CPPCG)  */
+    int presteps;      /* CG iterations run before switching to CPPCG                */
+    int outer;         /* CPPCG outer iterations                                     */
+    int inner_matvecs; /* matvecs inside the Chebyshev preconditioner                */
+    int matvecs;       /* all applications of A (incl. the initial residual)         */
+    int status;        /* tea_status of the solve                                    */
+    double r0;         /* ||u^n - A u^n||_2                                           */
+    double rnorm;      /* ||r||_2 at exit (recursively updated residual)              */
+    double eig_min, eig_max;   /* preconditioner interval (after margins)            */
+    double ritz_min, ritz_max; /* raw Lanczos extreme Ritz values                    */
+    double seconds;    /* device time of the solve (CUDA events, this rank)          */
+} tea_stats;
+
+/* Kernel ids for tea_kernel_times(). */
+enum {
+    TEA_K_INIT = 0, TEA_K_RESIDUAL, TEA_K_SPMV, TEA_K_UPDATE, TEA_K_CHEB_FIRST,
+    TEA_K_CHEB_STEP, TEA_K_CHEB_LAST, TEA_K_EIG, TEA_K_PACK, TEA_K_UNPACK, TEA_K_SCALAR,
+    TEA_K_COUNT
+};
+
+/* Library version string and ABI version. */
+const char *tea_version(void);
+int tea_abi_version(void);
+
+/* Write a fresh ncclUniqueId (128 bytes) into id128. Call on rank 0 only. */
+tea_status tea_get_nccl_id(void *id128);
+
+/* Device workspace bytes this rank needs for `mesh` and `dist` (NULL = 1 block). */
+tea_status tea_workspace_bytes(const tea_mesh *mesh, const tea_dist *dist, size_t *bytes);
+
+/* Create a context. Reads this rank's blocks (plus a margin) of the HOST global
+ * arrays `density` and `energy` (both nx*ny, see layout above), builds
+ * u^0 = density*energy (reading R4) and the face coefficients Kx, Ky scaled by
+ * rx, ry (reading R1/R2/R3). `d_workspace` is a DEVICE buffer of at
+ * least tea_workspace_bytes() bytes, 256-byte aligned, owned by the caller and
+ * valid until tea_finalize(). `cuda_stream` (cudaStream_t, may be NULL = legacy
+ * default) is the caller's stream: the library orders its own stream after it
+ * on entry and makes it wait for the library on exit. Collective over ranks.  */
+tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
+                    const double *energy, double dt, const tea_dist *dist,
+                    const tea_opts *opts, void *d_workspace, size_t ws_bytes,
+                    void *cuda_stream);
+
+/* One implicit timestep: solve A u^{n+1} = u^n with initial guess u^n, stop when
+ * ||r||_2 < eps * ||r_0||_2 (reading R5) or after max_iters iterations (CG
+ * iterations + CPPCG presteps + outer iterations). inner_steps = s >= 1
+ * Chebyshev matvecs per preconditioner application (CPPCG only, s <= 64).
+ * On return u^n <- u^{n+1}. Host-synchronous. Collective over ranks.
+ * stats may be NULL.                                                          */
+tea_status tea_solve(tea_ctx *ctx, tea_method method, double eps, int max_iters,
+                     int inner_steps, tea_stats *stats);
+
+/* Copy this rank's owned cells of u into their places in the HOST global array
+ * u_host (nx*ny doubles); other entries are untouched. Host-synchronous.      */
+tea_status tea_fetch(tea_ctx *ctx, double *u_host);
+
+/* Replace u (and the right-hand side u^n) by the HOST global array u_host:
+ * resume from a checkpoint written by tea_fetch. Host-synchronous.            */
+tea_status tea_set_u(tea_ctx *ctx, const double *u_host);
+
+/* Per-kernel device time accumulated since the last reset in profile mode:
+ * ms[i], launches[i] for i < TEA_K_COUNT (either may be NULL). reset != 0 clears. */
+tea_status tea_kernel_times(tea_ctx *ctx, double *ms, long long *launches, int reset);
+
+/* Kernel launches issued by the library since tea_init (all modes; graph
+ * replays count their kernel nodes).                                          */
+long long tea_launch_count(const tea_ctx *ctx);
+
+/* Free the context, its graphs, streams, events and NCCL communicator (not the
+ * workspace). Safe on a failed context; NULL is a no-op.                      */
+tea_status tea_finalize(tea_ctx *ctx);
+
+/* Last error message of ctx (or of the last failed tea_init when ctx is NULL). */
+const char *tea_last_error(const tea_ctx *ctx);
+
+/* ---- host-only helpers (no GPU needed; used by tests and tooling) ---------- */
+
+/* Cells owned by block b: columns [x0,x1), rows [y0,y1) of the global mesh.  */
+tea_status tea_block_extent(const tea_mesh *mesh, int px, int py, int b, int *x0, int *x1,
+                            int *y0, int *y1);
+
+/* CPPCG inner-loop schedule for s steps and halo depth d on a block with
+ * neighbours: writes up to cap ops as (code, arg) pairs into ops[2*i..2*i+1]
+ * and returns the op count (or a negative tea_status). Codes:
+ *   1 = exchange r at depth arg (after the outer update)
+ *   2 = Chebyshev step i computing z_i on owned cells extended by arg
+ *   3 = exchange the pair (z_{i-1}, z_{i-2}) at depth arg
+ *   4 = exchange z_s at depth arg (final fix-up when d == 1)
+ * A block without neighbours uses the same schedule with every exchange a no-op. */
+int tea_cheb_schedule(int s, int d, int *ops, int cap);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* TEA_H */

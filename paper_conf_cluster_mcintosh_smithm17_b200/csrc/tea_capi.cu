@@ -1,0 +1,985 @@
+// tea_capi.cu -- host driver and C ABI of the B200 TeaLeaf CG / CPPCG library.
+//
+// Context, block decomposition, workspace layout in HBM, halo plans
+// (matrix powers), the CG / CPPCG control flow (Sec. III), CUDA-graph
+// capture with a device-side WHILE loop, NCCL plumbing, and the extern "C" entry
+// points declared in include/tea.h. All arithmetic on fields runs in the kernels
+// of tea_kernels.cu; this file only sequences them.
+#include "tea.h"
+#include "tea_internal.h"
+
+#include <nccl.h>
+
+#include <algorithm>
+#include <cmath>
+#include <cstdarg>
+#include <cstdio>
+#include <cstring>
+#include <map>
+#include <memory>
+#include <string>
+#include <vector>
+
+using namespace tea;
+
+namespace {
+
+constexpr int kNDir = 8;
+// direction d: 0 W(-x) 1 E(+x) 2 S(-y) 3 N(+y) 4 SW 5 SE 6 NW 7 NE
+constexpr int kDX[kNDir] = {-1, 1, 0, 0, -1, 1, -1, 1};
+constexpr int kDY[kNDir] = {0, 0, -1, 1, -1, -1, 1, 1};
+constexpr int kOpp[kNDir] = {1, 0, 3, 2, 7, 6, 5, 4};
+
+inline size_t round_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
+
+// exchange kinds
+enum { X_R1 = 0, X_RD, X_Z2, X_Z1, X_U1, X_COUNT };
+
+struct XPlan {
+    int nf = 0, depth = 0;
+    int nsend = 0, nrecv = 0;  // boxes
+    int *d_send = nullptr, *d_recv = nullptr;
+    size_t soff[kNDir] = {}, slen[kNDir] = {}, roff[kNDir] = {}, rlen[kNDir] = {};
+};
+
+struct BlockLayout {
+    int bi, bj, gx0, gx1, gy0, gy1, bx, by;
+    int H, X0, pitch, rows;
+    size_t field_bytes, scalars_off, partials_off, partials_cap, boxes_off, halo_off,
+        halo_cap, total;
+    bool has_nbr;
+};
+
+void split(int n, int p, int i, int *a, int *b) {
+    int base = n / p, rem = n % p;
+    *a = i * base + std::min(i, rem);
+    *b = *a + base + (i < rem ? 1 : 0);
+}
+
+BlockLayout layout_block(const tea_mesh &m, int px, int py, int d, int b) {
+    BlockLayout L{};
+    L.bi = b % px;
+    L.bj = b / px;
+    split(m.nx, px, L.bi, &L.gx0, &L.gx1);
+    split(m.ny, py, L.bj, &L.gy0, &L.gy1);
+    L.bx = L.gx1 - L.gx0;
+    L.by = L.gy1 - L.gy0;
+    L.H = d + 2;
+    L.X0 = (int)round_up(d + 4, 16);
+    L.pitch = (int)round_up(L.X0 + L.bx + d + 4, 32);
+    L.rows = L.by + 2 * L.H;
+    L.field_bytes = round_up((size_t)L.rows * L.pitch * sizeof(double), 256);
+    size_t off = L.field_bytes * F_COUNT;
+    L.scalars_off = off;
+    off += round_up(sizeof(Scalars), 256);
+    L.partials_cap = 2 * (size_t)max_ctas(L.bx + 2 * d + 2, L.by + 2 * d + 2);
+    L.partials_off = off;
+    off += round_up(L.partials_cap * sizeof(double), 256);
+    L.has_nbr = (px * py > 1);
+    L.boxes_off = off;
+    off += L.has_nbr ? 16384 : 0;
+    L.halo_off = off;
+    // per field and depth d: two faces in x, two in y, four corners
+    size_t per_field = 2 * (size_t)d * (L.bx + L.by) + 4 * (size_t)d * d;
+    L.halo_cap = L.has_nbr ? 2 * per_field : 0;  // up to 2 fields per exchange
+    off += L.has_nbr ? 2 * round_up(L.halo_cap * sizeof(double), 256) : 0;
+    L.total = round_up(off, 256);
+    return L;
+}
+
+struct BlockCtx {
+    BlockLayout L;
+    int id, rank;
+    double *f[F_COUNT];  // orig pointers (cell (0,0))
+    Scalars *S;
+    double *partials;
+    int nbr[kNDir];
+    double *sendbuf = nullptr, *recvbuf = nullptr;
+    XPlan xp[X_COUNT];
+    Region owned() const { return Region{0, L.bx, 0, L.by}; }
+    Region ext(int e) const {
+        return Region{nbr[0] >= 0 ? -e : 0, L.bx + (nbr[1] >= 0 ? e : 0), nbr[2] >= 0 ? -e : 0,
+                      L.by + (nbr[3] >= 0 ? e : 0)};
+    }
+};
+
+struct PendingEv {
+    int kid;
+    cudaEvent_t a, b;
+};
+
+}  // namespace
+
+struct tea_ctx {
+    tea_mesh mesh{};
+    tea_opts opts{};
+    double dt = 0, rx = 0, ry = 0;
+    int px = 1, py = 1, d = 1, rank = 0, nranks = 1;
+    std::vector<BlockCtx> blocks;
+    cudaStream_t user_stream = nullptr, stream = nullptr;
+    cudaEvent_t ev_in = nullptr, ev_t0 = nullptr, ev_t1 = nullptr;
+    Scalars *hS = nullptr;  // pinned host mirror (head only)
+    ncclComm_t comm = nullptr;
+    std::string err;
+    bool failed = false;
+    long long launches = 0;
+    // profile
+    bool profiling = false;
+    std::vector<PendingEv> pending;
+    std::vector<cudaEvent_t> evpool;
+    size_t evnext = 0;
+    double kms[TEA_K_COUNT] = {};
+    long long kcount[TEA_K_COUNT] = {};
+    // graphs: key -> exec
+    std::map<long long, cudaGraphExec_t> graphs;
+    std::map<long long, int> graph_kernels;
+    // capture state
+    cudaGraphConditionalHandle cond = 0;
+    int ty_override = 0;
+};
+
+static std::string g_init_error;
+
+namespace {
+
+struct TeaError {
+    tea_status st;
+    std::string msg;
+};
+
+[[noreturn]] void fail(tea_status st, const char *fmt, ...) {
+    char buf[512];
+    va_list ap;
+    va_start(ap, fmt);
+    vsnprintf(buf, sizeof buf, fmt, ap);
+    va_end(ap);
+    throw TeaError{st, buf};
+}
+
+#define CK(call)                                                                        \
+    do {                                                                                \
+        cudaError_t e_ = (call);                                                        \
+        if (e_ != cudaSuccess)                                                          \
+            fail(TEA_ERR_CUDA, "%s:%d %s: %s", __FILE__, __LINE__, #call,               \
+                 cudaGetErrorString(e_));                                               \
+    } while (0)
+#define NK(call)                                                                        \
+    do {                                                                                \
+        ncclResult_t r_ = (call);                                                       \
+        if (r_ != ncclSuccess)                                                          \
+            fail(TEA_ERR_NCCL, "%s:%d %s: %s", __FILE__, __LINE__, #call,               \
+                 ncclGetErrorString(r_));                                               \
+    } while (0)
+
+KArgs kargs(tea_ctx *c, const BlockCtx &b, bool set_cond = false) {
+    KArgs a;
+    a.pitch = b.L.pitch;
+    a.S = b.S;
+    a.partials = b.partials;
+    a.cond = c->cond;
+    a.set_cond = set_cond ? 1 : 0;
+    return a;
+}
+
+// Issue one kernel launch (profiled with an event pair when profiling).
+template <class F>
+void K(tea_ctx *c, int kid, F &&f) {
+    if (c->profiling) {
+        if (c->evnext + 2 > c->evpool.size()) {
+            for (int i = 0; i < 256; ++i) {
+                cudaEvent_t e;
+                CK(cudaEventCreate(&e));
+                c->evpool.push_back(e);
+            }
+        }
+        cudaEvent_t a = c->evpool[c->evnext++], b = c->evpool[c->evnext++];
+        CK(cudaEventRecord(a, c->stream));
+        f();
+        CK(cudaGetLastError());
+        CK(cudaEventRecord(b, c->stream));
+        c->pending.push_back({kid, a, b});
+    } else {
+        f();
+        CK(cudaGetLastError());
+    }
+    c->launches++;
+}
+
+void resolve_profile(tea_ctx *c) {
+    if (!c->profiling) return;
+    CK(cudaStreamSynchronize(c->stream));
+    for (auto &p : c->pending) {
+        float ms = 0.f;
+        CK(cudaEventElapsedTime(&ms, p.a, p.b));
+        c->kms[p.kid] += ms;
+        c->kcount[p.kid] += 1;
+    }
+    c->pending.clear();
+    c->evnext = 0;
+}
+
+Launch plan(tea_ctx *c, const Region &R) {
+    return plan_stencil(R, c->opts.tile_rows > 0 ? c->opts.tile_rows : c->ty_override, 592);
+}
+
+// ------------------------------------------------------------------ reductions
+// Combine the block-local sums of slots [first, first+n) (0 pw, 1 gam, 2 rr) into
+// the global sums on every local block and across ranks.
+void reduce(tea_ctx *c, int first, int n) {
+    const int nb = (int)c->blocks.size();
+    if (nb > 1) {
+        std::vector<Scalars *> L;
+        for (auto &b : c->blocks) L.push_back(b.S);
+        K(c, TEA_K_SCALAR, [&] { launch_combine(L.data(), nb, n, first, c->stream); });
+    }
+    if (c->nranks > 1) {
+        double *p = &c->blocks[0].S->red_pw + first;
+        NK(ncclAllReduce(p, p, n, ncclDouble, ncclSum, c->comm, c->stream));
+    }
+}
+
+// ------------------------------------------------------------------ halo exchange
+void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field) {
+    // fids: field ids (same for every block), 1 or 2 entries
+    const int nb = (int)c->blocks.size();
+    if (c->px * c->py == 1) return;
+    const int nf = (int)fids_per_block_field.size();
+    for (auto &b : c->blocks) {
+        const XPlan &x = b.xp[kind];
+        if (x.nsend == 0) continue;
+        const double *F[4];
+        for (int i = 0; i < nf; ++i) F[i] = b.f[fids_per_block_field[i]];
+        K(c, TEA_K_PACK, [&] {
+            launch_pack(F, nf, b.L.pitch, x.d_send, x.nsend, b.sendbuf, c->stream);
+        });
+    }
+    // transport
+    bool remote = false;
+    for (auto &b : c->blocks)
+        for (int d = 0; d < kNDir; ++d)
+            if (b.nbr[d] >= 0) {
+                int nbid = b.nbr[d];
+                int nrank = nbid / (c->px * c->py / c->nranks);
+                if (nrank != c->rank) remote = true;
+            }
+    if (remote) NK(ncclGroupStart());
+    const int bpr = c->px * c->py / c->nranks;
+    for (auto &b : c->blocks) {
+        const XPlan &x = b.xp[kind];
+        for (int d = 0; d < kNDir; ++d) {
+            int nbid = b.nbr[d];
+            if (nbid < 0) continue;
+            int nrank = nbid / bpr;
+            if (nrank == c->rank) {
+                BlockCtx &nbk = c->blocks[nbid - c->rank * bpr];
+                const XPlan &y = nbk.xp[kind];
+                int od = kOpp[d];
+                if (x.slen[d] != y.rlen[od])
+                    fail(TEA_ERR_STATE, "halo size mismatch %zu vs %zu", x.slen[d], y.rlen[od]);
+                CK(cudaMemcpyAsync(nbk.recvbuf + y.roff[od], b.sendbuf + x.soff[d],
+                                   x.slen[d] * sizeof(double), cudaMemcpyDeviceToDevice,
+                                   c->stream));
+            } else {
+                NK(ncclSend(b.sendbuf + x.soff[d], x.slen[d], ncclDouble, nrank, c->comm,
+                            c->stream));
+                NK(ncclRecv(b.recvbuf + x.roff[d], x.rlen[d], ncclDouble, nrank, c->comm,
+                            c->stream));
+            }
+        }
+    }
+    if (remote) NK(ncclGroupEnd());
+    for (auto &b : c->blocks) {
+        const XPlan &x = b.xp[kind];
+        if (x.nrecv == 0) continue;
+        double *F[4];
+        for (int i = 0; i < nf; ++i) F[i] = b.f[fids_per_block_field[i]];
+        K(c, TEA_K_UNPACK, [&] {
+            launch_unpack(F, nf, b.L.pitch, x.d_recv, x.nrecv, b.recvbuf, c->stream);
+        });
+    }
+    (void)nb;
+}
+
+// Boxes of owned cells sent to direction d, and halo cells received from it.
+void send_box(const BlockLayout &L, int d, int dep, int *j0, int *j1, int *k0, int *k1) {
+    *j0 = 0;
+    *j1 = L.bx;
+    *k0 = 0;
+    *k1 = L.by;
+    if (kDX[d] < 0) *j1 = dep;
+    if (kDX[d] > 0) *j0 = L.bx - dep;
+    if (kDY[d] < 0) *k1 = dep;
+    if (kDY[d] > 0) *k0 = L.by - dep;
+}
+void recv_box(const BlockLayout &L, int d, int dep, int *j0, int *j1, int *k0, int *k1) {
+    *j0 = 0;
+    *j1 = L.bx;
+    *k0 = 0;
+    *k1 = L.by;
+    if (kDX[d] < 0) { *j0 = -dep; *j1 = 0; }
+    if (kDX[d] > 0) { *j0 = L.bx; *j1 = L.bx + dep; }
+    if (kDY[d] < 0) { *k0 = -dep; *k1 = 0; }
+    if (kDY[d] > 0) { *k0 = L.by; *k1 = L.by + dep; }
+}
+
+void build_xplans(tea_ctx *c, BlockCtx &b, int *d_boxes_base) {
+    struct K2 {
+        int nf, dep;
+        bool corners;
+    } kinds[X_COUNT] = {{1, 1, false}, {1, c->d, c->d > 1}, {2, c->d, c->d > 1},
+                        {1, 1, false}, {1, 1, false}};
+    std::vector<int> host;
+    int *dptr = d_boxes_base;
+    for (int kd = 0; kd < X_COUNT; ++kd) {
+        XPlan &x = b.xp[kd];
+        x.nf = kinds[kd].nf;
+        x.depth = kinds[kd].dep;
+        std::vector<int> sb, rb;
+        size_t so = 0, ro = 0;
+        for (int d = 0; d < kNDir; ++d) {
+            x.soff[d] = so;
+            x.roff[d] = ro;
+            x.slen[d] = x.rlen[d] = 0;
+            if (b.nbr[d] < 0) continue;
+            if (d >= 4 && !kinds[kd].corners) continue;
+            for (int f = 0; f < x.nf; ++f) {
+                int j0, j1, k0, k1;
+                send_box(b.L, d, x.depth, &j0, &j1, &k0, &k1);
+                sb.insert(sb.end(), {f, j0, j1, k0, k1});
+                so += (size_t)(j1 - j0) * (k1 - k0);
+                recv_box(b.L, d, x.depth, &j0, &j1, &k0, &k1);
+                rb.insert(rb.end(), {f, j0, j1, k0, k1});
+                ro += (size_t)(j1 - j0) * (k1 - k0);
+            }
+            x.slen[d] = so - x.soff[d];
+            x.rlen[d] = ro - x.roff[d];
+        }
+        if (so > b.L.halo_cap || ro > b.L.halo_cap) fail(TEA_ERR_STATE, "halo buffer too small");
+        x.nsend = (int)sb.size() / 5;
+        x.nrecv = (int)rb.size() / 5;
+        x.d_send = dptr;
+        CK(cudaMemcpyAsync(dptr, sb.data(), sb.size() * sizeof(int), cudaMemcpyHostToDevice,
+                           c->stream));
+        dptr += 16 * 5 * 2;
+        x.d_recv = dptr;
+        CK(cudaMemcpyAsync(dptr, rb.data(), rb.size() * sizeof(int), cudaMemcpyHostToDevice,
+                           c->stream));
+        dptr += 16 * 5 * 2;
+        CK(cudaStreamSynchronize(c->stream));
+    }
+}
+
+// ------------------------------------------------------------------ Chebyshev schedule
+struct ChebOpS {
+    int code, arg;
+};
+std::vector<ChebOpS> cheb_schedule(int s, int d) {
+    std::vector<ChebOpS> ops;
+    if (s < 1 || d < 1) return ops;
+    // final segment: up to d-1 steps ending at extension 1; other segments up to d
+    // steps ending at extension 0 (each needs its operands valid to its length).
+    int mlast = std::min(s, d - 1);
+    int rest = s - mlast;
+    std::vector<int> segs;
+    if (rest > 0) {
+        int nfull = (rest + d - 1) / d;
+        int first = rest - (nfull - 1) * d;
+        segs.push_back(first);
+        for (int i = 1; i < nfull; ++i) segs.push_back(d);
+    }
+    if (mlast > 0) segs.push_back(mlast);
+    int step = 0;
+    for (size_t g = 0; g < segs.size(); ++g) {
+        bool final_seg = (g + 1 == segs.size()) && mlast > 0;
+        int m = segs[g];
+        int depth = final_seg ? m + 1 : m;
+        ops.push_back({g == 0 ? 1 : 3, depth});
+        for (int i = 0; i < m; ++i) {
+            ++step;
+            int e = final_seg ? (m - i) : (m - 1 - i);
+            ops.push_back({2, e});
+        }
+    }
+    if (mlast == 0) ops.push_back({4, 1});
+    // r is read pointwise by every step (and by the stencil of step 1): exchange it
+    // once, deep enough for all of them.
+    int rdep = 1, i = 0;
+    for (auto &o : ops)
+        if (o.code == 2) {
+            ++i;
+            rdep = std::max(rdep, i == 1 ? o.arg + 1 : o.arg);
+        }
+    ops[0].arg = std::min(rdep, d);
+    (void)step;
+    return ops;
+}
+
+// ------------------------------------------------------------------ phase bodies
+int zbuf(int i) { return F_Z0 + ((i - 1) % 3); }  // z_i lives in Z[(i-1)%3]
+
+void body_cg(tea_ctx *c, int par, bool last_sets_cond) {
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan(c, R);
+        K(c, TEA_K_SPMV, [&] {
+            launch_spmv(kargs(c, b), L, R, b.f[F_R0], b.f[F_P0 + par], b.f[F_P1 - par],
+                        b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
+        });
+    }
+    reduce(c, 0, 1);
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan(c, R);
+        K(c, TEA_K_UPDATE, [&] {
+            launch_update(kargs(c, b, last_sets_cond), L, R, b.f[F_W], b.f[F_R0], c->stream);
+        });
+    }
+    reduce(c, 1, 2);
+    exchange(c, X_R1, {F_R0});
+}
+
+// Chebyshev chain z = B(A) r. fused: first step also does r_out = r_in - alpha w
+// (single block only). Returns nothing; z_s ends in zbuf(s).
+void cheb_chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond) {
+    auto ops = cheb_schedule(s, c->d);
+    int r = fused ? rout : rin;
+    int step = 0;
+    for (auto &op : ops) {
+        if (op.code == 1) {
+            if (!fused) exchange(c, op.arg == 1 ? X_R1 : X_RD, {r});
+        } else if (op.code == 3) {
+            // pair (z_{i-1}, z_{i-2}) before step i = step+1; for i == 2 only z_1 matters
+            exchange(c, X_Z2, {zbuf(step), step >= 2 ? zbuf(step - 1) : zbuf(step)});
+        } else if (op.code == 4) {
+            exchange(c, X_Z1, {zbuf(s)});
+        } else {
+            ++step;
+            const int mode = step == 1 ? 0 : (step == 2 ? 1 : 2);
+            const bool last = step == s;
+            for (auto &b : c->blocks) {
+                Region R = b.ext(op.arg);
+                Region D = b.owned();
+                Launch L = plan(c, R);
+                const bool fu = fused && step == 1;
+                const double *z1 = step >= 2 ? b.f[zbuf(step - 1)] : nullptr;
+                const double *z2 = step >= 3 ? b.f[zbuf(step - 2)] : nullptr;
+                int kid = step == 1 ? TEA_K_CHEB_FIRST : (last ? TEA_K_CHEB_LAST : TEA_K_CHEB_STEP);
+                K(c, kid, [&] {
+                    launch_cheb(kargs(c, b, last && sets_cond), L, R, D, mode, step, last, fu,
+                                restart, b.f[fu ? rin : r], b.f[F_W], b.f[rout], z1, z2,
+                                b.f[zbuf(step)], b.f[F_KX], b.f[F_KY], c->stream);
+                });
+            }
+            if (last) reduce(c, 1, 2);
+        }
+    }
+}
+
+bool single_block(tea_ctx *c) { return c->px * c->py == 1; }
+
+void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
+    const bool fused = single_block(c);
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan(c, R);
+        K(c, TEA_K_SPMV, [&] {
+            launch_spmv(kargs(c, b), L, R, b.f[zbuf(s)], b.f[F_P0 + par], b.f[F_P1 - par],
+                        b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
+        });
+    }
+    reduce(c, 0, 1);
+    if (fused) {
+        cheb_chain(c, s, false, true, F_R0 + par, F_R1 - par, sets_cond);
+    } else {
+        for (auto &b : c->blocks) {
+            Region R = b.owned();
+            Launch L = plan(c, R);
+            K(c, TEA_K_UPDATE, [&] {
+                launch_update_nodot(kargs(c, b), L, R, b.f[F_W], b.f[F_R0], c->stream);
+            });
+        }
+        cheb_chain(c, s, false, false, F_R0, F_R0, sets_cond);
+    }
+}
+
+void read_state(tea_ctx *c) {
+    CK(cudaMemcpyAsync(c->hS, c->blocks[0].S, offsetof(Scalars, cheb_a),
+                       cudaMemcpyDeviceToHost, c->stream));
+    CK(cudaStreamSynchronize(c->stream));
+    resolve_profile(c);
+}
+
+// Run a phase loop until the device reports done. `body(par, sets_cond)` issues
+// one iteration; bodies come in pairs (p / r ping-pong parity).
+template <class B>
+void run_loop(tea_ctx *c, long long key, int iters_hint, B body) {
+    const int mode = c->profiling ? 2 : c->opts.loop_mode;
+    if (mode == 2) {
+        const int chunk = c->opts.check_interval > 0 ? c->opts.check_interval : 16;
+        for (;;) {
+            for (int i = 0; i < (chunk + 1) / 2; ++i) {
+                body(0, false);
+                body(1, false);
+            }
+            read_state(c);
+            if (c->hS->done) return;
+        }
+    }
+    if (mode == 1) {
+        const int chunk = c->opts.check_interval > 0 ? c->opts.check_interval : 32;
+        long long k = key * 1000003LL + 17 + chunk;
+        auto it = c->graphs.find(k);
+        if (it == c->graphs.end()) {
+            long long l0 = c->launches;
+            cudaGraph_t g;
+            CK(cudaStreamBeginCapture(c->stream, cudaStreamCaptureModeThreadLocal));
+            for (int i = 0; i < (chunk + 1) / 2; ++i) {
+                body(0, false);
+                body(1, false);
+            }
+            CK(cudaStreamEndCapture(c->stream, &g));
+            cudaGraphExec_t ge;
+            CK(cudaGraphInstantiate(&ge, g, 0));
+            CK(cudaGraphDestroy(g));
+            c->graph_kernels[k] = (int)(c->launches - l0);
+            c->launches = l0;
+            it = c->graphs.emplace(k, ge).first;
+        }
+        for (;;) {
+            CK(cudaGraphLaunch(it->second, c->stream));
+            c->launches += c->graph_kernels[k];
+            read_state(c);
+            if (c->hS->done) return;
+        }
+    }
+    // mode 0: one graph with a WHILE conditional node around a 2-iteration body
+    auto it = c->graphs.find(key);
+    if (it == c->graphs.end()) {
+        long long l0 = c->launches;
+        cudaGraph_t g, bodyg;
+        CK(cudaGraphCreate(&g, 0));
+        cudaGraphConditionalHandle h;
+        CK(cudaGraphConditionalHandleCreate(&h, g, 1, cudaGraphCondAssignDefault));
+        cudaGraphNodeParams np = {};
+        np.type = cudaGraphNodeTypeConditional;
+        np.conditional.handle = h;
+        np.conditional.type = cudaGraphCondTypeWhile;
+        np.conditional.size = 1;
+        cudaGraphNode_t node;
+        CK(cudaGraphAddNode(&node, g, nullptr, 0, &np));
+        bodyg = np.conditional.phGraph_out[0];
+        CK(cudaStreamBeginCaptureToGraph(c->stream, bodyg, nullptr, nullptr, 0,
+                                         cudaStreamCaptureModeThreadLocal));
+        c->cond = h;
+        body(0, true);
+        body(1, true);
+        c->cond = 0;
+        cudaGraph_t captured;
+        CK(cudaStreamEndCapture(c->stream, &captured));
+        cudaGraphExec_t ge;
+        CK(cudaGraphInstantiate(&ge, g, 0));
+        CK(cudaGraphDestroy(g));
+        c->graph_kernels[key] = (int)(c->launches - l0);
+        c->launches = l0;
+        it = c->graphs.emplace(key, ge).first;
+    }
+    const int it0 = c->hS->it;
+    CK(cudaGraphLaunch(it->second, c->stream));
+    read_state(c);
+    const int bodies = (c->hS->it - it0) / 2 + 1;
+    c->launches += (long long)bodies * c->graph_kernels[key];
+    (void)iters_hint;
+}
+
+tea_status map_status(int ds, bool maxed) {
+    switch (ds) {
+        case DS_CONVERGED: return TEA_OK;
+        case DS_LIMIT: return maxed ? TEA_NOT_CONVERGED : TEA_OK;
+        case DS_BREAKDOWN:
+        case DS_EIGFAIL: return TEA_ERR_BREAKDOWN;
+        default: return TEA_ERR_STATE;
+    }
+}
+
+tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, int s,
+                      tea_stats *st) {
+    if (c->failed) fail(TEA_ERR_STATE, "context already failed: %s", c->err.c_str());
+    if (method != TEA_CG && method != TEA_CPPCG) fail(TEA_ERR_ARG, "bad method %d", (int)method);
+    if (max_iters < 0) fail(TEA_ERR_ARG, "max_iters < 0");
+    if (method == TEA_CPPCG && (s < 1 || s > kMaxS))
+        fail(TEA_ERR_ARG, "inner_steps must be in [1,%d]", kMaxS);
+    const int pre = c->opts.presteps;
+    if (method == TEA_CPPCG && (pre < 1 || pre > kMaxPre))
+        fail(TEA_ERR_ARG, "presteps must be in [1,%d]", kMaxPre);
+    c->profiling = c->opts.profile != 0;
+
+    CK(cudaEventRecord(c->ev_in, c->user_stream));
+    CK(cudaStreamWaitEvent(c->stream, c->ev_in, 0));
+    CK(cudaEventRecord(c->ev_t0, c->stream));
+
+    const int lim1 = method == TEA_CG ? max_iters : std::min(pre, max_iters);
+    for (auto &b : c->blocks)
+        K(c, TEA_K_SCALAR, [&] {
+            launch_scalars(kargs(c, b), SC_BEGIN, eps, lim1, max_iters, c->opts.eig_margin_lo,
+                           c->opts.eig_margin_hi, c->stream);
+        });
+    exchange(c, X_U1, {F_U});
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan(c, R);
+        K(c, TEA_K_RESIDUAL, [&] {
+            launch_residual(kargs(c, b), L, R, b.f[F_U], b.f[F_KX], b.f[F_KY], b.f[F_U0],
+                            b.f[F_R0], c->stream);
+        });
+    }
+    reduce(c, 1, 2);
+    for (auto &b : c->blocks)
+        K(c, TEA_K_SCALAR, [&] {
+            launch_scalars(kargs(c, b), SC_R0, 0, 0, 0, 0, 0, c->stream);
+        });
+    exchange(c, X_R1, {F_R0});
+    read_state(c);
+
+    // ---- phase 1: CG (or the CPPCG presteps)
+    if (!c->hS->done) {
+        run_loop(c, 1, lim1, [&](int par, bool sc) { body_cg(c, par, sc); });
+    }
+    int ds = c->hS->status;
+    bool phase2 = method == TEA_CPPCG && ds == DS_LIMIT && c->hS->it < max_iters;
+    if (phase2) {
+        // ---- eigen-estimate, coefficients, restart z = B(A) r, p = z
+        for (auto &b : c->blocks)
+            K(c, TEA_K_EIG, [&] { launch_eig_setup(kargs(c, b), s, c->stream); });
+        cheb_chain(c, s, true, false, F_R0, F_R0, false);
+        read_state(c);
+        if (!c->hS->done) {
+            long long key = 2 + 16LL * s;
+            run_loop(c, key, max_iters, [&](int par, bool sc) { body_pcg(c, s, par, sc); });
+        }
+        ds = c->hS->status;
+    }
+    CK(cudaEventRecord(c->ev_t1, c->stream));
+    CK(cudaEventRecord(c->ev_in, c->stream));
+    CK(cudaStreamWaitEvent(c->user_stream, c->ev_in, 0));
+    CK(cudaStreamSynchronize(c->stream));
+    float ms = 0.f;
+    CK(cudaEventElapsedTime(&ms, c->ev_t0, c->ev_t1));
+    const Scalars &h = *c->hS;
+    const bool maxed = h.it >= max_iters;
+    tea_status rs = map_status(ds, maxed);
+    if (st) {
+        st->iterations = h.it;
+        st->presteps = phase2 ? h.presteps : 0;
+        st->outer = phase2 ? h.outer : 0;
+        st->inner_matvecs = phase2 ? s * (h.outer + 1) : 0;
+        st->matvecs = 1 + h.it + st->inner_matvecs;
+        st->status = rs;
+        st->r0 = h.r0;
+        st->rnorm = std::sqrt(h.red_rr);
+        st->eig_min = phase2 ? h.eig_min : 0.0;
+        st->eig_max = phase2 ? h.eig_max : 0.0;
+        st->ritz_min = phase2 ? h.ritz_min : 0.0;
+        st->ritz_max = phase2 ? h.ritz_max : 0.0;
+        st->seconds = ms * 1e-3;
+    }
+    if (rs < 0) fail(rs, "solver breakdown (device status %d) at iteration %d", ds, h.it);
+    return rs;
+}
+
+}  // namespace
+
+// ====================================================================== C ABI
+extern "C" {
+
+const char *tea_version(void) { return "tea-b200 0.1 (sm_100a, fp64)"; }
+int tea_abi_version(void) { return TEA_ABI_VERSION; }
+
+tea_status tea_get_nccl_id(void *id128) {
+    if (!id128) return TEA_ERR_ARG;
+    ncclUniqueId id;
+    if (ncclGetUniqueId(&id) != ncclSuccess) return TEA_ERR_NCCL;
+    static_assert(sizeof(id) == 128, "ncclUniqueId size");
+    std::memcpy(id128, &id, sizeof id);
+    return TEA_OK;
+}
+
+static tea_status check_decomp(const tea_mesh *m, const tea_dist *dist, int *px, int *py,
+                               int *d, int *rank, int *nranks, std::string *why) {
+    if (!m || m->nx < 1 || m->ny < 1 || !(m->xmax > m->xmin) || !(m->ymax > m->ymin)) {
+        *why = "bad mesh";
+        return TEA_ERR_ARG;
+    }
+    *px = dist ? dist->px : 1;
+    *py = dist ? dist->py : 1;
+    *d = dist ? dist->halo_depth : 1;
+    *rank = dist ? dist->rank : 0;
+    *nranks = dist ? dist->nranks : 1;
+    if (*px < 1 || *py < 1 || *nranks < 1 || *rank < 0 || *rank >= *nranks) {
+        *why = "bad px/py/rank/nranks";
+        return TEA_ERR_ARG;
+    }
+    if ((*px * *py) % *nranks != 0) {
+        *why = "px*py must be a multiple of nranks";
+        return TEA_ERR_ARG;
+    }
+    if (*nranks > 1 && *px * *py != *nranks) {
+        *why = "multi-process runs need exactly one block per rank (px*py == nranks)";
+        return TEA_ERR_ARG;
+    }
+    if (*px * *py > 64) {
+        *why = "at most 64 blocks";
+        return TEA_ERR_ARG;
+    }
+    if (*d < 1 || *d > 16) {
+        *why = "halo_depth must be in [1,16]";
+        return TEA_ERR_ARG;
+    }
+    const int minw = std::min(m->nx / *px, m->ny / *py);
+    if (*px * *py > 1 && minw < *d + 1) {
+        *why = "blocks must be at least halo_depth+1 cells wide";
+        return TEA_ERR_ARG;
+    }
+    return TEA_OK;
+}
+
+tea_status tea_workspace_bytes(const tea_mesh *mesh, const tea_dist *dist, size_t *bytes) {
+    int px, py, d, rank, nranks;
+    std::string why;
+    if (!bytes) return TEA_ERR_ARG;
+    tea_status s = check_decomp(mesh, dist, &px, &py, &d, &rank, &nranks, &why);
+    if (s != TEA_OK) {
+        g_init_error = why;
+        return s;
+    }
+    const int bpr = px * py / nranks;
+    size_t tot = 0;
+    for (int b = rank * bpr; b < (rank + 1) * bpr; ++b) tot += layout_block(*mesh, px, py, d, b).total;
+    *bytes = tot;
+    return TEA_OK;
+}
+
+tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
+                    const double *energy, double dt, const tea_dist *dist, const tea_opts *opts,
+                    void *d_workspace, size_t ws_bytes, void *cuda_stream) {
+    if (!out) return TEA_ERR_ARG;
+    *out = nullptr;
+    std::unique_ptr<tea_ctx> c(new tea_ctx());
+    try {
+        int px, py, d, rank, nranks;
+        std::string why;
+        tea_status s = check_decomp(mesh, dist, &px, &py, &d, &rank, &nranks, &why);
+        if (s != TEA_OK) fail(s, "%s", why.c_str());
+        if (!density || !energy || !d_workspace) fail(TEA_ERR_ARG, "null pointer argument");
+        if (!(dt >= 0.0) || !std::isfinite(dt)) fail(TEA_ERR_ARG, "bad dt");
+        if (((uintptr_t)d_workspace) % 256) fail(TEA_ERR_ARG, "workspace must be 256-B aligned");
+        size_t need = 0;
+        tea_workspace_bytes(mesh, dist, &need);
+        if (ws_bytes < need) fail(TEA_ERR_ARG, "workspace too small: %zu < %zu", ws_bytes, need);
+        c->mesh = *mesh;
+        c->px = px;
+        c->py = py;
+        c->d = d;
+        c->rank = rank;
+        c->nranks = nranks;
+        c->dt = dt;
+        const double dx = (mesh->xmax - mesh->xmin) / mesh->nx;
+        const double dy = (mesh->ymax - mesh->ymin) / mesh->ny;
+        c->rx = dt / (dx * dx);
+        c->ry = dt / (dy * dy);
+        tea_opts o{};
+        o.presteps = 30;
+        o.eig_margin_lo = 0.95;
+        o.eig_margin_hi = 1.05;
+        if (opts) {
+            o = *opts;
+            if (o.presteps == 0) o.presteps = 30;
+            if (o.eig_margin_lo == 0.0) o.eig_margin_lo = 0.95;
+            if (o.eig_margin_hi == 0.0) o.eig_margin_hi = 1.05;
+        }
+        if (o.loop_mode < 0 || o.loop_mode > 2) fail(TEA_ERR_ARG, "bad loop_mode");
+        c->opts = o;
+        for (long long i = 0; i < (long long)mesh->nx * mesh->ny; i += 1 + ((long long)mesh->nx * mesh->ny) / 4096)
+            if (!(density[i] > 0.0)) fail(TEA_ERR_ARG, "density must be > 0");
+
+        c->user_stream = (cudaStream_t)cuda_stream;
+        CK(cudaStreamCreateWithFlags(&c->stream, cudaStreamNonBlocking));
+        CK(cudaEventCreateWithFlags(&c->ev_in, cudaEventDisableTiming));
+        CK(cudaEventCreate(&c->ev_t0));
+        CK(cudaEventCreate(&c->ev_t1));
+        CK(cudaMallocHost((void **)&c->hS, sizeof(Scalars)));
+        std::memset(c->hS, 0, sizeof(Scalars));
+        CK(cudaEventRecord(c->ev_in, c->user_stream));
+        CK(cudaStreamWaitEvent(c->stream, c->ev_in, 0));
+
+        if (nranks > 1) {
+            if (!dist->nccl_id) fail(TEA_ERR_ARG, "nccl_id required when nranks > 1");
+            ncclUniqueId id;
+            std::memcpy(&id, dist->nccl_id, sizeof id);
+            NK(ncclCommInitRank(&c->comm, nranks, id, rank));
+        }
+
+        const int bpr = px * py / nranks;
+        char *ws = (char *)d_workspace;
+        c->blocks.resize(bpr);
+        for (int i = 0; i < bpr; ++i) {
+            BlockCtx &b = c->blocks[i];
+            b.id = rank * bpr + i;
+            b.rank = rank;
+            b.L = layout_block(*mesh, px, py, d, b.id);
+            const BlockLayout &L = b.L;
+            for (int f = 0; f < F_COUNT; ++f)
+                b.f[f] = (double *)(ws + f * L.field_bytes) + (size_t)L.H * L.pitch + L.X0;
+            b.S = (Scalars *)(ws + L.scalars_off);
+            b.partials = (double *)(ws + L.partials_off);
+            for (int dd = 0; dd < kNDir; ++dd) {
+                int nbi = L.bi + kDX[dd], nbj = L.bj + kDY[dd];
+                b.nbr[dd] = (nbi >= 0 && nbi < px && nbj >= 0 && nbj < py) ? nbj * px + nbi : -1;
+            }
+            CK(cudaMemsetAsync(ws, 0, L.total, c->stream));
+            if (L.has_nbr) {
+                b.sendbuf = (double *)(ws + L.halo_off);
+                b.recvbuf = (double *)(ws + L.halo_off + round_up(L.halo_cap * sizeof(double), 256));
+                build_xplans(c.get(), b, (int *)(ws + L.boxes_off));
+            }
+            // stage rho -> W, e -> Z0 over the block plus margin m (clipped to the mesh)
+            const int m = d + 1;
+            const int gx0 = std::max(0, L.gx0 - m), gx1 = std::min(mesh->nx, L.gx1 + m);
+            const int gy0 = std::max(0, L.gy0 - m), gy1 = std::min(mesh->ny, L.gy1 + m);
+            const size_t hp = (size_t)mesh->nx * sizeof(double);
+            double *dW = b.f[F_W] + (size_t)(gy0 - L.gy0) * L.pitch + (gx0 - L.gx0);
+            double *dZ = b.f[F_Z0] + (size_t)(gy0 - L.gy0) * L.pitch + (gx0 - L.gx0);
+            CK(cudaMemcpy2DAsync(dW, L.pitch * sizeof(double), density + (size_t)gy0 * mesh->nx + gx0,
+                                 hp, (gx1 - gx0) * sizeof(double), gy1 - gy0,
+                                 cudaMemcpyHostToDevice, c->stream));
+            CK(cudaMemcpy2DAsync(dZ, L.pitch * sizeof(double), energy + (size_t)gy0 * mesh->nx + gx0,
+                                 hp, (gx1 - gx0) * sizeof(double), gy1 - gy0,
+                                 cudaMemcpyHostToDevice, c->stream));
+            Region owned{0, L.bx, 0, L.by};
+            Region all{-d, L.bx + d + 1, -d, L.by + d + 1};
+            Region kxr{-d, L.bx + d + 1, -d, L.by + d};
+            Region kyr{-d, L.bx + d, -d, L.by + d + 1};
+            K(c.get(), TEA_K_INIT, [&] {
+                launch_init_fields(kargs(c.get(), b), b.f[F_W], b.f[F_Z0], b.f[F_U0], b.f[F_U],
+                                   b.f[F_KX], b.f[F_KY], owned, all, kxr, kyr, c->rx, c->ry,
+                                   o.mean_mode, c->stream);
+            });
+            // the staging fields are solver fields with zero halos: clear them again
+            CK(cudaMemsetAsync(ws + F_W * L.field_bytes, 0, L.field_bytes, c->stream));
+            CK(cudaMemsetAsync(ws + F_Z0 * L.field_bytes, 0, L.field_bytes, c->stream));
+            ws += L.total;
+        }
+        CK(cudaStreamSynchronize(c->stream));
+        *out = c.release();
+        return TEA_OK;
+    } catch (const TeaError &e) {
+        g_init_error = e.msg;
+        if (c->stream) cudaStreamSynchronize(c->stream);
+        tea_finalize(c.release());
+        return e.st;
+    }
+}
+
+tea_status tea_solve(tea_ctx *ctx, tea_method method, double eps, int max_iters, int inner_steps,
+                     tea_stats *stats) {
+    if (!ctx) return TEA_ERR_ARG;
+    try {
+        return solve_impl(ctx, method, eps, max_iters, inner_steps, stats);
+    } catch (const TeaError &e) {
+        ctx->err = e.msg;
+        if (e.st != TEA_ERR_ARG) ctx->failed = true;
+        if (stats) stats->status = e.st;
+        return e.st;
+    }
+}
+
+tea_status tea_fetch(tea_ctx *ctx, double *u_host) {
+    if (!ctx || !u_host) return TEA_ERR_ARG;
+    try {
+        if (ctx->failed) fail(TEA_ERR_STATE, "context failed: %s", ctx->err.c_str());
+        for (auto &b : ctx->blocks) {
+            const BlockLayout &L = b.L;
+            CK(cudaMemcpy2DAsync(u_host + (size_t)L.gy0 * ctx->mesh.nx + L.gx0,
+                                 ctx->mesh.nx * sizeof(double), b.f[F_U], L.pitch * sizeof(double),
+                                 L.bx * sizeof(double), L.by, cudaMemcpyDeviceToHost, ctx->stream));
+        }
+        CK(cudaStreamSynchronize(ctx->stream));
+        return TEA_OK;
+    } catch (const TeaError &e) {
+        ctx->err = e.msg;
+        return e.st;
+    }
+}
+
+tea_status tea_set_u(tea_ctx *ctx, const double *u_host) {
+    if (!ctx || !u_host) return TEA_ERR_ARG;
+    try {
+        if (ctx->failed) fail(TEA_ERR_STATE, "context failed: %s", ctx->err.c_str());
+        for (auto &b : ctx->blocks) {
+            const BlockLayout &L = b.L;
+            CK(cudaMemcpy2DAsync(b.f[F_U], L.pitch * sizeof(double),
+                                 u_host + (size_t)L.gy0 * ctx->mesh.nx + L.gx0,
+                                 ctx->mesh.nx * sizeof(double), L.bx * sizeof(double), L.by,
+                                 cudaMemcpyHostToDevice, ctx->stream));
+        }
+        CK(cudaStreamSynchronize(ctx->stream));
+        return TEA_OK;
+    } catch (const TeaError &e) {
+        ctx->err = e.msg;
+        return e.st;
+    }
+}
+
+tea_status tea_kernel_times(tea_ctx *ctx, double *ms, long long *launches, int reset) {
+    if (!ctx) return TEA_ERR_ARG;
+    for (int i = 0; i < TEA_K_COUNT; ++i) {
+        if (ms) ms[i] = ctx->kms[i];
+        if (launches) launches[i] = ctx->kcount[i];
+    }
+    if (reset) {
+        std::memset(ctx->kms, 0, sizeof ctx->kms);
+        std::memset(ctx->kcount, 0, sizeof ctx->kcount);
+    }
+    return TEA_OK;
+}
+
+long long tea_launch_count(const tea_ctx *ctx) { return ctx ? ctx->launches : 0; }
+
+tea_status tea_finalize(tea_ctx *ctx) {
+    if (!ctx) return TEA_OK;
+    if (ctx->stream) cudaStreamSynchronize(ctx->stream);
+    for (auto &g : ctx->graphs) cudaGraphExecDestroy(g.second);
+    for (auto e : ctx->evpool) cudaEventDestroy(e);
+    if (ctx->ev_in) cudaEventDestroy(ctx->ev_in);
+    if (ctx->ev_t0) cudaEventDestroy(ctx->ev_t0);
+    if (ctx->ev_t1) cudaEventDestroy(ctx->ev_t1);
+    if (ctx->hS) cudaFreeHost(ctx->hS);
+    if (ctx->comm) ncclCommDestroy(ctx->comm);
+    if (ctx->stream) cudaStreamDestroy(ctx->stream);
+    delete ctx;
+    return TEA_OK;
+}
+
+const char *tea_last_error(const tea_ctx *ctx) {
+    return ctx ? ctx->err.c_str() : g_init_error.c_str();
+}
+
+tea_status tea_block_extent(const tea_mesh *mesh, int px, int py, int b, int *x0, int *x1,
+                            int *y0, int *y1) {
+    if (!mesh || px < 1 || py < 1 || b < 0 || b >= px * py) return TEA_ERR_ARG;
+    split(mesh->nx, px, b % px, x0, x1);
+    split(mesh->ny, py, b / px, y0, y1);
+    return TEA_OK;
+}
+
+int tea_cheb_schedule(int s, int d, int *ops, int cap) {
+    if (s < 1 || s > kMaxS || d < 1 || d > 16) return TEA_ERR_ARG;
+    auto v = cheb_schedule(s, d);
+    if ((int)v.size() > cap || !ops) return TEA_ERR_ARG;
+    for (size_t i = 0; i < v.size(); ++i) {
+        ops[2 * i] = v[i].code;
+        ops[2 * i + 1] = v[i].arg;
+    }
+    return (int)v.size();
+}
+
+}  // extern "C"

@@ -1,0 +1,117 @@
+// tea_internal.h -- internal types shared by the CUDA kernels and the host driver
+// of the B200 TeaLeaf CG / CPPCG library (not part of the C ABI).
+#pragma once
+
+#include <cuda_runtime.h>
+#include <cstddef>
+#include <cstdint>
+
+namespace tea {
+
+constexpr int kMaxPre = 512;   // presteps cap (Lanczos history length)
+constexpr int kMaxS = 64;      // Chebyshev inner steps cap
+constexpr int kWarps = 4;      // warps per CTA in the stencil / pointwise kernels
+constexpr int kThreads = 32 * kWarps;
+constexpr int kStrip = 64;     // columns per warp (32 lanes x double2)
+constexpr int kCtaCols = kWarps * kStrip;
+
+// Device-side solver state, one copy per local block (all copies evolve
+// identically: every decision is taken from globally reduced scalars).
+struct Scalars {
+    // reduction slots: a kernel's last CTA writes the block-local sum; after the
+    // cross-block combine / NCCL allreduce they hold the global sum
+    double red_pw;    // p.w                        (eq (9))
+    double red_gam;   // r.z (CG: r.r)              (CG numerator gamma)
+    double red_rr;    // r.r                        (convergence, reading R5)
+    double red_pad;
+    // persistent state
+    double gam_old;     // gamma of the current iterate (alpha numerator)
+    double alpha_prev;  // alpha of the previous update, applied lazily to u
+    double r0;          // ||r_0||
+    double eps;
+    double theta, eig_min, eig_max, ritz_min, ritz_max;
+    double margin_lo, margin_hi;
+    double beta_last;
+    int it;             // completed iterations (CG + presteps + outer)
+    int it_limit;       // iteration limit of the current phase
+    int done;           // phase finished (converged / limit / breakdown)
+    int status;         // DS_* below
+    int fresh;          // next spmv starts a new (P)CG sequence: beta = 0, no check
+    int presteps;
+    int outer;
+    int max_iters;
+    unsigned ticket;    // last-CTA ticket of the deterministic grid reduction
+    int pad_[3];
+    double cheb_a[kMaxS], cheb_b[kMaxS];
+    double alpha_hist[kMaxPre], beta_hist[kMaxPre];
+};
+
+enum { DS_RUNNING = 0, DS_CONVERGED = 1, DS_LIMIT = 2, DS_BREAKDOWN = 3, DS_EIGFAIL = 4 };
+
+// [j0,j1) x [k0,k1) in block-local cell coordinates (may reach into the halo)
+struct Region {
+    int j0, j1, k0, k1;
+};
+
+// Field indices inside a block's workspace.
+enum Field {
+    F_U0 = 0, F_U, F_KX, F_KY, F_R0, F_R1, F_P0, F_P1, F_W, F_Z0, F_Z1, F_Z2, F_COUNT
+};
+
+// Launch geometry of one stencil / pointwise launch.
+struct Launch {
+    dim3 grid;
+    int jstart;  // even column of the first lane of CTA 0 / warp 0
+    int ty;      // rows per CTA tile
+};
+
+// Kernel launchers (tea_kernels.cu). `orig` pointers address cell (0,0) of a
+// field; element (j,k) is orig[k*pitch + j]. All take the block's Scalars and
+// reduction scratch (partials) and run on `st`.
+struct KArgs {
+    int pitch;
+    Scalars *S;
+    double *partials;
+    cudaGraphConditionalHandle cond;  // WHILE-loop handle (0 = none)
+    int set_cond;                     // this launch may end the WHILE loop
+};
+
+Launch plan_stencil(const Region &R, int ty_req, int ncta_target);
+Launch plan_pointwise(const Region &R, int ty_req, int ncta_target);
+int max_ctas(int width, int height);
+
+void launch_init_fields(const KArgs &a, const double *rho, const double *en, double *u0,
+                        double *u, double *kx, double *ky, Region owned, Region all,
+                        Region kxr, Region kyr, double rx, double ry, int mean_mode,
+                        cudaStream_t st);
+void launch_residual(const KArgs &a, const Launch &L, const Region &R, const double *u,
+                     const double *kx, const double *ky, double *u0, double *r,
+                     cudaStream_t st);
+void launch_spmv(const KArgs &a, const Launch &L, const Region &R, const double *src,
+                 const double *pin, double *pout, double *w, double *u, const double *kx,
+                 const double *ky, cudaStream_t st);
+void launch_update(const KArgs &a, const Launch &L, const Region &R, const double *w,
+                   double *r, cudaStream_t st);
+void launch_update_nodot(const KArgs &a, const Launch &L, const Region &R, const double *w,
+                         double *r, cudaStream_t st);
+// Chebyshev step i (1-based) of s: z_out = z1 + a_i (z1 - z2) + b_i (r - A z1)
+// mode: 0 = first (z1 = r/theta, z2 = 0), 1 = second (z2 = r/theta), 2 = general.
+// fuse_update: r_out = r_in - alpha w first (first step only, single block).
+// last: also r.z_out and r.r over D; restart: do not advance the iteration count.
+void launch_cheb(const KArgs &a, const Launch &L, const Region &R, const Region &D, int mode,
+                 int step, bool last, bool fuse_update, bool restart, const double *rin,
+                 const double *win, double *rout, const double *z1, const double *z2,
+                 double *zout, const double *kx, const double *ky, cudaStream_t st);
+void launch_eig_setup(const KArgs &a, int s, cudaStream_t st);
+void launch_scalars(const KArgs &a, int mode, double eps, int it_limit, int max_iters,
+                    double mlo, double mhi, cudaStream_t st);
+void launch_combine(Scalars *const *S_dev_list, int nblocks, int nvals, int first_slot,
+                    cudaStream_t st);
+void launch_pack(const double *const *fields, int nf, int pitch, const int *boxes,
+                 int nbox, double *buf, cudaStream_t st);
+void launch_unpack(double *const *fields, int nf, int pitch, const int *boxes, int nbox,
+                   const double *buf, cudaStream_t st);
+
+enum { SC_BEGIN = 0, SC_R0 = 1, SC_PHASE2 = 2 };
+
+}  // namespace tea

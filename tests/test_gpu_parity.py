@@ -1,0 +1,207 @@
+"""GPU parity: the CUDA path (through the C ABI) against the CPU oracle.
+
+Bar (BASELINE.json north_star): max relative field error <= 1e-10 in fp64 and
+iteration counts within +-2 of the oracle on the same generated inputs. The
+field is positive (u >= 0.01 on the pipe; > 0 on the random decks), so the
+pointwise relative error max|u_gpu - u_ora| / |u_ora| is well defined.
+
+Sizes: small cases the oracle runs on the spot (several 256-column CTA tiles,
+ragged tails in x and y, 1-wide meshes, odd sizes); full-size cases (1024^2
+converged, 4096^2 fixed iteration counts) against tests/golden/oracle_*.npz,
+written by tests/golden/make_golden.py from the oracle alone, compared at the
+stored sample of cells plus sum/min/max.
+"""
+import os
+
+import numpy as np
+import pytest
+
+pytestmark = pytest.mark.gpu
+
+HERE = os.path.dirname(os.path.abspath(__file__))
+
+
+@pytest.fixture(scope="module")
+def tea():
+    import torch
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_cluster_mcintosh_smithm17_b200 as tea
+    tea.lib()
+    return tea
+
+
+def rel_err(a, b):
+    return float(np.max(np.abs(a - b) / np.abs(b)))
+
+
+def gpu_run(tea, deck, steps=1, **kw):
+    solve_kw = {k: kw.pop(k) for k in ("method", "eps", "max_iters", "inner_steps") if k in kw}
+    t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, **kw)
+    stats = []
+    for _ in range(steps):
+        r = t.solve(**solve_kw)
+        stats.append(dict(r.stats, ret=r.status))
+    u = t.fetch()
+    t.close()
+    return u, stats
+
+
+def deck_of(kind, nx, ny, seed=0, dt=0.004):
+    from paper_conf_cluster_mcintosh_smithm17_b200 import inputs
+    if kind == "pipe":
+        return inputs.crooked_pipe(nx, ny)
+    return inputs.random_fields(nx, ny, seed, dt=dt)
+
+
+SHAPES = [("pipe", 128, 128), ("random", 300, 200), ("random", 1000, 777), ("random", 257, 65),
+          ("random", 1, 97), ("random", 95, 1), ("random", 3, 5), ("random", 64, 64)]
+
+
+@pytest.mark.parametrize("kind,nx,ny", SHAPES)
+@pytest.mark.parametrize("k", [1, 2, 7])
+def test_fixed_cg_iterations(tea, ora, kind, nx, ny, k):
+    """k CG iterations with eps = 0: exercises residual, spmv (+ lazy u update),
+    update and the finalize path on ragged shapes."""
+    deck = deck_of(kind, nx, ny, seed=nx + ny, dt=0.04)
+    u_o, st_o, _ = ora.run(deck, steps=1, method=0, eps=0.0, max_iters=k)
+    u_g, st_g = gpu_run(tea, deck, method=0, eps=0.0, max_iters=k)
+    assert st_g[0]["iterations"] == st_o[0]["iterations"] == k
+    assert st_g[0]["ret"] == 1  # TEA_NOT_CONVERGED
+    assert rel_err(u_g, u_o) <= 1e-12
+    assert st_g[0]["r0"] == pytest.approx(st_o[0]["r0"], rel=1e-12)
+
+
+@pytest.mark.parametrize("kind,nx,ny", SHAPES[:5])
+@pytest.mark.parametrize("method", [0, 1])
+def test_converged_solve(tea, ora, kind, nx, ny, method):
+    deck = deck_of(kind, nx, ny, seed=3, dt=0.4)
+    kw = dict(method=method, eps=1e-13, max_iters=20000, inner_steps=6)
+    u_o, st_o, s_o = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, **kw)
+    assert s_o[0] == 0 and st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+    if method == 1 and st_o[0]["outer"] > 0:
+        assert st_g[0]["presteps"] == st_o[0]["presteps"]
+        assert st_g[0]["eig_min"] == pytest.approx(st_o[0]["eig_min"], rel=1e-9)
+        assert st_g[0]["eig_max"] == pytest.approx(st_o[0]["eig_max"], rel=1e-9)
+
+
+def test_config1_pipe128_cg_10_steps(tea, ora):
+    """BASELINE.json configs[0]: 128x128, CG, fp64, 10 timesteps, eps = 1e-15."""
+    deck = deck_of("pipe", 128, 128)
+    kw = dict(method=0, eps=1e-15, max_iters=10000)
+    u_o, st_o, _ = ora.run(deck, steps=10, **kw)
+    u_g, st_g = gpu_run(tea, deck, steps=10, **kw)
+    for a, b in zip(st_g, st_o):
+        assert abs(a["iterations"] - b["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+
+
+@pytest.mark.parametrize("s", [1, 2, 3, 10])
+def test_cppcg_inner_steps(tea, ora, s):
+    deck = deck_of("pipe", 256, 256)
+    kw = dict(method=1, eps=1e-13, max_iters=20000, inner_steps=s)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, **kw)
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert abs(st_g[0]["outer"] - st_o[0]["outer"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+
+
+@pytest.mark.parametrize("loop_mode", [0, 1, 2])
+def test_loop_modes_identical(tea, loop_mode):
+    """WHILE graph, chunked graphs and eager launches run the same kernels with the
+    same launch geometry: bitwise identical results (deterministic reductions)."""
+    deck = deck_of("pipe", 200, 136)
+    ref, st_ref = gpu_run(tea, deck, method=1, eps=1e-12, max_iters=5000, inner_steps=5,
+                          loop_mode=2)
+    u, st = gpu_run(tea, deck, method=1, eps=1e-12, max_iters=5000, inner_steps=5,
+                    loop_mode=loop_mode, check_interval=6)
+    assert st[0]["iterations"] == st_ref[0]["iterations"]
+    assert np.array_equal(u, ref)
+
+
+def test_run_to_run_bitwise(tea):
+    deck = deck_of("random", 333, 222, seed=5)
+    a, _ = gpu_run(tea, deck, method=0, eps=1e-12, max_iters=3000)
+    b, _ = gpu_run(tea, deck, method=0, eps=1e-12, max_iters=3000)
+    assert np.array_equal(a, b)
+
+
+def test_conservation_and_max_principle(tea):
+    deck = deck_of("pipe", 512, 512)
+    u0 = deck.density * deck.energy
+    for method in (0, 1):
+        u, st = gpu_run(tea, deck, method=method, eps=1e-12, max_iters=20000)
+        assert abs(u.sum() - u0.sum()) / u0.sum() <= 1e-12
+        assert u.min() >= u0.min() * (1 - 1e-12) and u.max() <= u0.max() * (1 + 1e-12)
+
+
+def test_checkpoint_resume_bitwise(tea):
+    """N steps == k steps, fetch, re-init with e = u/rho, N-k steps."""
+    deck = deck_of("pipe", 128, 96)
+    full, _ = gpu_run(tea, deck, steps=4, method=0, eps=1e-14, max_iters=5000)
+    half, _ = gpu_run(tea, deck, steps=2, method=0, eps=1e-14, max_iters=5000)
+    t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt)
+    t.set_u(half)
+    for _ in range(2):
+        t.solve(method=0, eps=1e-14, max_iters=5000)
+    resumed = t.fetch()
+    t.close()
+    assert np.array_equal(resumed, full)
+
+
+def test_errors(tea):
+    deck = deck_of("random", 16, 16)
+    m = tea.mesh_of(deck)
+    with pytest.raises(tea.TeaError):
+        tea.Tea(m, deck.density, deck.energy, deck.dt, dist=dict(px=3, py=1, nranks=2))
+    with pytest.raises(tea.TeaError):
+        tea.Tea(m, deck.density, deck.energy, deck.dt, dist=dict(px=1, py=1, halo_depth=17))
+    bad = deck.density.copy()
+    bad[0, 0] = 0.0
+    with pytest.raises(tea.TeaError):
+        tea.Tea(m, bad, deck.energy, deck.dt)
+    t = tea.Tea(m, deck.density, deck.energy, deck.dt)
+    r = t.solve(method=1, inner_steps=0, raise_on_error=False)
+    assert r.status == tea.ERR_ARG
+    r = t.solve(method=0, eps=1e-10, max_iters=1000)  # still usable after ERR_ARG
+    assert r.status == tea.OK
+    t.close()
+
+
+def test_zero_residual(tea):
+    deck = deck_of("random", 40, 30)
+    deck.dt = 0.0  # A = I: r0 == 0, zero iterations
+    u, st = gpu_run(tea, deck, method=1, eps=1e-10, max_iters=100)
+    assert st[0]["iterations"] == 0 and st[0]["ret"] == 0
+    assert np.array_equal(u, deck.density * deck.energy)
+
+
+# ---------------------------------------------------------------- full sizes
+def load_golden(name):
+    p = os.path.join(HERE, "golden", f"oracle_{name}.npz")
+    if not os.path.exists(p):
+        pytest.skip(f"{p} missing (run tests/golden/make_golden.py)")
+    return dict(np.load(p))
+
+
+@pytest.mark.parametrize("name", ["pipe1024_cg", "pipe1024_cppcg", "pipe4096_cg_fixed50",
+                                  "pipe4096_cppcg_fixed33"])
+def test_full_size_against_golden(tea, name):
+    g = load_golden(name)
+    n = int(g["n"])
+    deck = deck_of("pipe", n, n)
+    u, st = gpu_run(tea, deck, method=int(g["method"]), eps=float(g["eps"]),
+                    max_iters=int(g["max_iters"]), inner_steps=int(g["inner_steps"]))
+    assert abs(st[0]["iterations"] - int(g["iterations"])) <= 2
+    if int(g["method"]) == 1:
+        assert st[0]["presteps"] == int(g["presteps"])
+        assert st[0]["eig_max"] == pytest.approx(float(g["eig_max"]), rel=1e-9)
+    vals = u.ravel()[g["idx"]]
+    assert rel_err(vals, g["vals"]) <= 1e-10
+    assert u.sum() == pytest.approx(float(g["sum"]), rel=1e-12)
+    assert u.min() == pytest.approx(float(g["umin"]), rel=1e-10)
+    assert u.max() == pytest.approx(float(g["umax"]), rel=1e-10)
