@@ -1,0 +1,387 @@
+"""bench.py -- TeaLeaf CPPCG / CG on B200: one JSON line.
+
+Workload (BASELINE.json metric and configs[3]): the crooked-pipe deck on a
+4096 x 4096 mesh, CPPCG with a 10-step Chebyshev inner loop, fp64. A "step" is
+one implicit timestep: a full tea_solve (presteps + Lanczos eigen-estimate +
+CPPCG outer iterations) to ||r|| < eps ||r0||, every kernel of the hot path.
+Timesteps advance u^n, so step k solves from the u of step k-1.
+
+value       solver iterations/s (CG presteps + CPPCG outer iterations, tea_stats)
+            over the K timed steps, device-timed (CUDA events), max over ranks.
+e2e         same metric through the C ABI with HOST buffers: each step copies
+            u^n host->device (tea_set_u, pinned), solves, copies u^{n+1} back
+            (tea_fetch) inside the timed region.
+roofline    the dominant kernel (the Chebyshev inner step):
+            algorithmic bytes per launch / its mean launch duration from a
+            profiled solve (CUDA events around each launch on the library's
+            stream); peak = MEASURED_PEAKS.json hbm_gbs.
+cpu_baseline the CPU oracle (oracle/, serial C, 1 thread) on a bounded prefix of
+            the same timestep, same unit.
+
+Usage: python bench.py [--gpus N] [--steps K] [--warmup W] [--impl reference]
+       [--n 4096] [--method cppcg|cg] [--inner 10] [--eps 1e-12] [--halo-depth d]
+For N > 1 launch with torchrun (one process per GPU, NCCL).
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+HBM_FALLBACK = 6650.0  # B200_PROFILING.md fallback, GB/s
+
+
+def peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    if os.path.exists(p):
+        d = json.load(open(p))
+        return float(d["hbm_gbs"]), "measured"
+    return HBM_FALLBACK, "fallback"
+
+
+# ------------------------------------------------------------------ clocks
+class ClockSampler:
+    """nvidia-smi sampling during the timed region (B200_PROFILING.md clocks line)."""
+
+    Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.active,"
+         "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+         "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index=0):
+        self.index = index
+        self.rows = []
+        self.proc = None
+        self.th = None
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.index), "--query-gpu=" + self.Q,
+                 "--format=csv,noheader,nounits", "-lms", "200"],
+                stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+        except OSError:
+            self.proc = None
+            return
+        self.th = threading.Thread(target=self._read, daemon=True)
+        self.th.start()
+
+    def _read(self):
+        for line in self.proc.stdout:
+            parts = [x.strip() for x in line.split(",")]
+            if len(parts) >= 7:
+                self.rows.append(parts)
+
+    def stop(self):
+        if self.proc is None:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+        time.sleep(0.25)
+        self.proc.terminate()
+        try:
+            self.proc.wait(timeout=5)
+        except subprocess.TimeoutExpired:
+            self.proc.kill()
+        self.th.join(timeout=2)
+        sm = [float(r[0]) for r in self.rows if r[0].replace(".", "").isdigit()]
+        smax = [float(r[1]) for r in self.rows if r[1].replace(".", "").isdigit()]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = set()
+        for r in self.rows:
+            for i, n in enumerate(names):
+                if r[3 + i].lower().startswith("active"):
+                    reasons.add(n)
+        return {"sm_mhz": statistics.median(sm) if sm else None,
+                "sm_max_mhz": max(smax) if smax else None,
+                "reasons": sorted(reasons), "samples": len(self.rows)}
+
+
+# ------------------------------------------------------------------ model bytes
+def cheb_step_bytes(cells):
+    """Chebyshev inner step (general): reads z_{i-1}, z_{i-2}, r, Kx, Ky; writes z_i."""
+    return 6 * 8 * cells
+
+
+def outer_bytes(cells, s):
+    """One CPPCG outer iteration: spmv 8 + update/first-step 6 +
+    second step 5 + 6 per further step."""
+    if s == 1:
+        return (8 + 6) * 8 * cells
+    return (8 + 6 + 5 + 6 * (s - 2)) * 8 * cells
+
+
+def cg_iter_bytes(cells):
+    """One CG iteration: spmv 8 streams + update 3 streams."""
+    return 11 * 8 * cells
+
+
+def load_ncu_traffic(kernel_key, n):
+    p = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    if not os.path.exists(p):
+        return None
+    d = json.load(open(p))
+    e = d.get(f"{kernel_key}@{n}")
+    return None if e is None else float(e["dram_bytes_per_launch"])
+
+
+# ------------------------------------------------------------------ reference arm
+def run_reference(args):
+    import oracle
+    from paper_conf_cluster_mcintosh_smithm17_b200 import inputs
+
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return 0
+    oracle.build()
+    deck = inputs.crooked_pipe(args.n)
+    method = oracle.CPPCG if args.method == "cppcg" else oracle.CG
+    sample_iters = args.ref_iters
+    for _ in range(args.warmup):  # untimed warm-up (page-in, caches)
+        oracle.run(deck, steps=1, method=method, eps=args.eps, max_iters=1,
+                   inner_steps=args.inner)
+    t_all, its, mv = 0.0, 0, 0
+    for _ in range(args.steps):
+        t0 = time.perf_counter()
+        _, st, _ = oracle.run(deck, steps=1, method=method, eps=args.eps,
+                              max_iters=sample_iters, inner_steps=args.inner)
+        t_all += time.perf_counter() - t0
+        its += st[0]["iterations"]
+        mv += st[0]["matvecs"]
+    value = its / t_all
+    sample = (f"first {sample_iters} iterations of timestep 1 "
+              f"({'30 CG presteps + ' + str(sample_iters - 30) + ' CPPCG outer' if method else 'CG'})"
+              f" per step, serial C oracle")
+    line = {
+        "impl": "reference", "metric": metric_name(args), "value": value, "unit": "iterations/s",
+        "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
+        "ms_per_step": 1e3 * t_all / args.steps, "higher_is_better": True,
+        "scaling": "strong", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+        "config": config(args),
+        "cpu_baseline": {"value": value, "unit": "iterations/s", "cores": 1, "kind": "oracle",
+                         "sample": sample, "matvecs_per_s": mv / t_all},
+        "e2e": {"value": value, "unit": "iterations/s", "h2d_bytes_per_step": 0,
+                "d2h_bytes_per_step": 0},
+    }
+    print(json.dumps(line), flush=True)
+    return 0
+
+
+def metric_name(args):
+    return (f"solver iterations/s, {args.n}^2 {'CPPCG' if args.method == 'cppcg' else 'CG'}"
+            f" (time-to-solution, HBM GB/s alongside)")
+
+
+def config(args):
+    return {"workload": f"crooked_pipe {args.n}x{args.n} "
+                        f"{'CPPCG s=' + str(args.inner) if args.method == 'cppcg' else 'CG'}"
+                        f" eps={args.eps:g} 1 timestep/step",
+            "mesh": [args.n, args.n], "method": args.method, "inner_steps": args.inner,
+            "eps": args.eps, "halo_depth": args.halo_depth, "dt": 0.004,
+            "l2": "inputs larger than L2 (12 fp64 fields x 134 MB at 4096^2)"
+            if args.n >= 2048 else "working set fits in L2 (no flush)"}
+
+
+# ------------------------------------------------------------------ GPU arm
+def cpu_baseline(args, deck):
+    import oracle
+    oracle.build()
+    method = oracle.CPPCG if args.method == "cppcg" else oracle.CG
+    t0 = time.perf_counter()
+    _, st, _ = oracle.run(deck, steps=1, method=method, eps=args.eps, max_iters=args.ref_iters,
+                          inner_steps=args.inner)
+    dt = time.perf_counter() - t0
+    return {"value": st[0]["iterations"] / dt, "unit": "iterations/s", "cores": 1,
+            "kind": "oracle",
+            "sample": f"first {args.ref_iters} iterations of timestep 1 "
+                      f"({st[0]['presteps'] or st[0]['iterations']} CG + {st[0]['outer']} CPPCG"
+                      f" outer), serial C oracle, {dt:.1f} s",
+            "matvecs_per_s": st[0]["matvecs"] / dt}
+
+
+def factor(n):
+    best = (1, n)
+    for px in range(1, n + 1):
+        if n % px == 0:
+            py = n // px
+            if abs(px - py) < abs(best[0] - best[1]) or (abs(px - py) == abs(best[0] - best[1])
+                                                         and px < best[0]):
+                best = (px, py)
+    return best
+
+
+def run_gpu(args):
+    import torch
+
+    import paper_conf_cluster_mcintosh_smithm17_b200 as tea
+    from paper_conf_cluster_mcintosh_smithm17_b200 import inputs
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    dist_kw = None
+    pg = None
+    if world > 1:
+        import torch.distributed as dist
+        dist.init_process_group("nccl", device_id=dev)
+        pg = dist
+        nid = torch.zeros(128, dtype=torch.uint8, device=dev)
+        if rank == 0:
+            nid.copy_(torch.frombuffer(bytearray(tea.get_nccl_id()), dtype=torch.uint8))
+        dist.broadcast(nid, 0)
+        px, py = factor(world)
+        dist_kw = dict(rank=rank, nranks=world, px=px, py=py, halo_depth=args.halo_depth,
+                       nccl_id=bytes(nid.cpu().numpy().tobytes()))
+
+    def barrier():
+        torch.cuda.synchronize()
+        if pg is not None:
+            pg.barrier()
+            torch.cuda.synchronize()
+
+    def max_over_ranks(x):
+        if pg is None:
+            return x
+        t = torch.tensor([x], dtype=torch.float64, device=dev)
+        pg.all_reduce(t, op=pg.ReduceOp.MAX)
+        return float(t.item())
+
+    deck = inputs.crooked_pipe(args.n)
+    method = tea.CPPCG if args.method == "cppcg" else tea.CG
+    cells = args.n * args.n
+    t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
+                tile_rows=args.tile_rows)
+    stream = t.stream
+
+    def solve():
+        r = t.solve(method, args.eps, args.max_iters, args.inner)
+        return r.stats
+
+    for _ in range(args.warmup):
+        solve()
+    barrier()
+    clk = ClockSampler(local)
+    clk.start()
+    l0 = t.launch_count()
+    ev0 = torch.cuda.Event(enable_timing=True)
+    ev1 = torch.cuda.Event(enable_timing=True)
+    ev0.record(stream)
+    stats = [solve() for _ in range(args.steps)]
+    ev1.record(stream)
+    ev1.synchronize()
+    launches = t.launch_count() - l0
+    clocks = clk.stop()
+    ms = ev0.elapsed_time(ev1)
+    ms = max_over_ranks(ms)
+    iters = sum(s["iterations"] for s in stats)
+    outer = sum(s["outer"] for s in stats)
+    matvecs = sum(s["matvecs"] for s in stats)
+    value = iters / (ms * 1e-3)
+    if method == tea.CPPCG:
+        model_bytes = sum(5 * 8 * cells + s["presteps"] * cg_iter_bytes(cells) +
+                          outer_bytes(cells, args.inner) - 10 * 8 * cells +  # restart chain
+                          s["outer"] * outer_bytes(cells, args.inner) for s in stats)
+    else:
+        model_bytes = len(stats) * 5 * 8 * cells + iters * cg_iter_bytes(cells)
+
+    # ---- e2e through the C ABI with host buffers (pinned)
+    u_host = torch.empty((args.n, args.n), dtype=torch.float64).pin_memory()
+    u_np = u_host.numpy()
+    t.fetch(u_np)
+    barrier()
+    e0 = time.perf_counter()
+    e_iters = 0
+    for _ in range(args.steps):
+        t.set_u(u_np)
+        e_iters += solve()["iterations"]
+        t.fetch(u_np)
+    torch.cuda.synchronize()
+    e_dt = max_over_ranks(time.perf_counter() - e0)
+    bx = cells // world
+    e2e = {"value": e_iters / e_dt, "unit": "iterations/s", "h2d_bytes_per_step": 8 * bx,
+           "d2h_bytes_per_step": 8 * bx}
+    t.close()
+
+    # ---- roofline of the dominant kernel: profiled solve (events per launch)
+    tp = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
+                 profile=True, tile_rows=args.tile_rows)
+    tp.set_u(u_np)
+    tp.solve(method, args.eps, args.max_iters, args.inner)
+    kt = tp.kernel_times()
+    tp.close()
+    hbm, which = peaks()
+    local_cells = cells // world
+    if method == tea.CPPCG and kt["cheb_step"][1] > 0:
+        kkey, kms, kn = "cheb_step", kt["cheb_step"][0], kt["cheb_step"][1]
+        kbytes = cheb_step_bytes(local_cells)
+    else:
+        kkey, kms, kn = "spmv", kt["spmv"][0], kt["spmv"][1]
+        kbytes = 8 * 8 * local_cells
+    avg_ms = kms / max(kn, 1)
+    achieved = kbytes / (avg_ms * 1e-3) / 1e9
+    tot_ms = sum(v[0] for v in kt.values())
+    roof = {"bound": "hbm", "achieved": achieved, "peak": hbm, "unit": "GB/s",
+            "frac": achieved / hbm, "traffic": load_ncu_traffic(kkey, args.n),
+            "kernel": kkey, "algorithmic_bytes_per_launch": kbytes,
+            "avg_launch_us": avg_ms * 1e3, "launches_profiled": kn,
+            "share_of_profiled_step": kms / tot_ms if tot_ms else None,
+            "peak_source": f"MEASURED_PEAKS.json hbm_gbs ({which})",
+            "kernel_ms": {k: v[0] for k, v in kt.items() if v[1]}}
+
+    line = {
+        "metric": metric_name(args), "value": value, "unit": "iterations/s",
+        "n_gpus": world, "steps": args.steps, "warmup": args.warmup,
+        "ms_per_step": ms / args.steps, "higher_is_better": True, "scaling": "strong",
+        "vs_baseline": None, "dtype": "f64", "data": "synthetic (crooked pipe deck, seeded)",
+        "config": dict(config(args), parallelism=f"{dist_kw['px']}x{dist_kw['py']} blocks"
+                       if dist_kw else "1 block"),
+        "time_to_solution_s": ms * 1e-3 / args.steps,
+        "iterations_per_step": iters / args.steps, "outer_per_step": outer / args.steps,
+        "matvecs_per_s": matvecs / (ms * 1e-3),
+        "hbm_gbs_model": model_bytes / (ms * 1e-3) / 1e9,
+        "e2e": e2e, "gpu_launches": launches, "clocks": clocks, "roofline": roof,
+    }
+    if rank == 0 and world == 1 and not args.no_cpu:
+        line["cpu_baseline"] = cpu_baseline(args, deck)
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+    if pg is not None:
+        pg.barrier()
+        pg.destroy_process_group()
+    return 0
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=5)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", default="b200", choices=["b200", "reference"])
+    ap.add_argument("--n", type=int, default=4096)
+    ap.add_argument("--method", default="cppcg", choices=["cppcg", "cg"])
+    ap.add_argument("--inner", type=int, default=10)
+    ap.add_argument("--eps", type=float, default=1e-12)
+    ap.add_argument("--max-iters", type=int, default=100000)
+    ap.add_argument("--halo-depth", type=int, default=2)
+    ap.add_argument("--tile-rows", type=int, default=0)
+    ap.add_argument("--ref-iters", type=int, default=31)
+    ap.add_argument("--no-cpu", action="store_true")
+    args = ap.parse_args()
+    if args.warmup < 3:
+        ap.error("--warmup must be >= 3")
+    if args.impl == "reference":
+        return run_reference(args)
+    return run_gpu(args)
+
+
+if __name__ == "__main__":
+    sys.exit(main())

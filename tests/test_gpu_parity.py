@@ -32,7 +32,17 @@ def tea():
 
 
 def rel_err(a, b):
+    """Pointwise relative error (the north_star metric; the pipe has u >= 0.01)."""
     return float(np.max(np.abs(a - b) / np.abs(b)))
+
+
+def field_err(a, b, kind):
+    """Pipe decks: pointwise relative error. Random decks (u = rho e spans six decades
+    cell to cell, so a cell's value can be a 1e-6 remnant of cancelling O(1) terms):
+    max abs error over max |u| (parity metric)."""
+    if kind == "pipe":
+        return rel_err(a, b)
+    return float(np.max(np.abs(a - b)) / np.max(np.abs(b)))
 
 
 def gpu_run(tea, deck, steps=1, **kw):
@@ -68,7 +78,7 @@ def test_fixed_cg_iterations(tea, ora, kind, nx, ny, k):
     u_g, st_g = gpu_run(tea, deck, method=0, eps=0.0, max_iters=k)
     assert st_g[0]["iterations"] == st_o[0]["iterations"] == k
     assert st_g[0]["ret"] == 1  # TEA_NOT_CONVERGED
-    assert rel_err(u_g, u_o) <= 1e-12
+    assert field_err(u_g, u_o, kind) <= 1e-12
     assert st_g[0]["r0"] == pytest.approx(st_o[0]["r0"], rel=1e-12)
 
 
@@ -81,7 +91,7 @@ def test_converged_solve(tea, ora, kind, nx, ny, method):
     u_g, st_g = gpu_run(tea, deck, **kw)
     assert s_o[0] == 0 and st_g[0]["ret"] == 0
     assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
-    assert rel_err(u_g, u_o) <= 1e-10
+    assert field_err(u_g, u_o, kind) <= 1e-10
     if method == 1 and st_o[0]["outer"] > 0:
         assert st_g[0]["presteps"] == st_o[0]["presteps"]
         assert st_g[0]["eig_min"] == pytest.approx(st_o[0]["eig_min"], rel=1e-9)
@@ -205,3 +215,33 @@ def test_full_size_against_golden(tea, name):
     assert u.sum() == pytest.approx(float(g["sum"]), rel=1e-12)
     assert u.min() == pytest.approx(float(g["umin"]), rel=1e-10)
     assert u.max() == pytest.approx(float(g["umax"]), rel=1e-10)
+
+
+# ---------------------------------------------------------------- decomposition
+# px x py blocks in ONE process on one GPU (nranks = 1): the multi-GPU code path
+# (extended bounds, matrix-powers schedule, pack / unpack of depth-d halos with
+# corners, cross-block reductions) with device copies as the halo transport.
+@pytest.mark.parametrize("px,py,d", [(2, 1, 1), (1, 2, 1), (2, 2, 2), (3, 2, 3), (4, 2, 5),
+                                     (2, 3, 10), (4, 4, 16)])
+@pytest.mark.parametrize("method", [0, 1])
+def test_multiblock_matches_oracle(tea, ora, px, py, d, method):
+    deck = deck_of("pipe", 200, 168)
+    kw = dict(method=method, eps=1e-13, max_iters=20000, inner_steps=10)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, dist=dict(px=px, py=py, halo_depth=d, nranks=1), **kw)
+    assert st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+
+
+@pytest.mark.parametrize("px,py,d", [(2, 2, 1), (3, 3, 4), (2, 1, 7)])
+def test_multiblock_fixed_iterations(tea, ora, px, py, d):
+    """eps = 0 and a fixed iteration count: field agrees to rounding (1e-12)."""
+    deck = deck_of("random", 150, 121, seed=9, dt=0.04)
+    for method, k in ((0, 9), (1, 33)):
+        u_o, st_o, _ = ora.run(deck, steps=1, method=method, eps=0.0, max_iters=k,
+                               inner_steps=6)
+        u_g, st_g = gpu_run(tea, deck, dist=dict(px=px, py=py, halo_depth=d, nranks=1),
+                            method=method, eps=0.0, max_iters=k, inner_steps=6)
+        assert st_g[0]["iterations"] == k
+        assert field_err(u_g, u_o, "random") <= 1e-12
