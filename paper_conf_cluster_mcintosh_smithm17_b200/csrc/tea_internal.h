@@ -42,7 +42,8 @@ struct Scalars {
     int max_iters;
     unsigned ticket;    // last-CTA ticket of the deterministic grid reduction
     int pad_[3];
-    double cheb_a[kMaxS], cheb_b[kMaxS];
+    double cheb_a[kMaxS], cheb_b[kMaxS];                 // Saad 12.1 a_i, b_i
+    double cheb_cx[kMaxS], cheb_cz[kMaxS], cheb_cr[kMaxS], cheb_ca[kMaxS];  // folded, §4.3
     double alpha_hist[kMaxPre], beta_hist[kMaxPre];
 };
 

@@ -85,7 +85,10 @@ def test_fixed_cg_iterations(tea, ora, kind, nx, ny, k):
 @pytest.mark.parametrize("kind,nx,ny", SHAPES[:5])
 @pytest.mark.parametrize("method", [0, 1])
 def test_converged_solve(tea, ora, kind, nx, ny, method):
-    deck = deck_of(kind, nx, ny, seed=3, dt=0.4)
+    # dt = 0.004 (the deck's): kappa ~ 1e3-1e4. At kappa ~ 1e6 (dt = 0.4, 3700 CG
+    # iterations) CG's finite-precision iteration count drifts by ~10 between any two
+    # summation orders, so +-2 is not a meaningful bar there.
+    deck = deck_of(kind, nx, ny, seed=3, dt=0.004)
     kw = dict(method=method, eps=1e-13, max_iters=20000, inner_steps=6)
     u_o, st_o, s_o = ora.run(deck, steps=1, **kw)
     u_g, st_g = gpu_run(tea, deck, **kw)
