@@ -219,7 +219,7 @@ void resolve_profile(tea_ctx *c) {
 }
 
 Launch plan(tea_ctx *c, const Region &R) {
-    return plan_stencil(R, c->opts.tile_rows > 0 ? c->opts.tile_rows : c->ty_override, 592);
+    return plan_stencil(R, c->opts.tile_rows > 0 ? c->opts.tile_rows : c->ty_override, 1184);
 }
 
 // ------------------------------------------------------------------ reductions
