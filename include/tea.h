@@ -80,6 +80,10 @@ typedef struct {
     int check_interval;     /* iterations per chunk in loop_mode 1/2 (0 = auto) [0]    */
     int profile;            /* 1: eager launches timed per kernel (tea_kernel_times)[0]*/
     int tile_rows;          /* rows per CTA tile of the stencil kernels, 0 = auto [0]  */
+    int tb_steps;           /* Chebyshev steps fused per HBM pass (on-chip matrix
+                               powers, single block only): 0 = auto, 1 = one kernel
+                               per step, 2..5 = at most that many            [0 = 4] */
+    int tb_rows;            /* output rows per CTA tile of the fused passes, 0 = auto */
 } tea_opts;
 
 /* Per-solve statistics. */
@@ -101,6 +105,7 @@ typedef struct {
 enum {
     TEA_K_INIT = 0, TEA_K_RESIDUAL, TEA_K_SPMV, TEA_K_UPDATE, TEA_K_CHEB_FIRST,
     TEA_K_CHEB_STEP, TEA_K_CHEB_LAST, TEA_K_EIG, TEA_K_PACK, TEA_K_UNPACK, TEA_K_SCALAR,
+    TEA_K_TB_FIRST, TEA_K_TB_MID, TEA_K_TB_LAST, /* fused multi-step Chebyshev passes */
     TEA_K_COUNT
 };
 
@@ -144,9 +149,13 @@ tea_status tea_fetch(tea_ctx *ctx, double *u_host);
  * resume from a checkpoint written by tea_fetch. Host-synchronous.            */
 tea_status tea_set_u(tea_ctx *ctx, const double *u_host);
 
-/* Per-kernel device time accumulated since the last reset in profile mode:
- * ms[i], launches[i] for i < TEA_K_COUNT (either may be NULL). reset != 0 clears. */
-tea_status tea_kernel_times(tea_ctx *ctx, double *ms, long long *launches, int reset);
+/* Per-kernel-class device time accumulated since the last reset in profile mode:
+ * ms[i], launches[i] and bytes[i] for i < TEA_K_COUNT (any may be NULL). bytes are
+ * the ALGORITHMIC HBM bytes of those launches (fp64 streams x 8 B x owned cells, the
+ * model of DESIGN.md §4; halos and redundant overlap compute excluded).
+ * reset != 0 clears.                                                           */
+tea_status tea_kernel_times(tea_ctx *ctx, double *ms, long long *launches, double *bytes,
+                            int reset);
 
 /* Kernel launches issued by the library since tea_init (all modes; graph
  * replays count their kernel nodes).                                          */

@@ -24,7 +24,7 @@ CG, CPPCG = 0, 1
 OK, NOT_CONVERGED = 0, 1
 ERR_ARG, ERR_CUDA, ERR_NCCL, ERR_BREAKDOWN, ERR_STATE = -1, -2, -3, -4, -5
 KERNELS = ["init", "residual", "spmv", "update", "cheb_first", "cheb_step", "cheb_last", "eig",
-           "pack", "unpack", "scalar"]
+           "pack", "unpack", "scalar", "tb_first", "tb_mid", "tb_last"]
 SYMBOLS = ["tea_version", "tea_abi_version", "tea_get_nccl_id", "tea_workspace_bytes", "tea_init",
            "tea_solve", "tea_fetch", "tea_set_u", "tea_kernel_times", "tea_launch_count",
            "tea_finalize", "tea_last_error", "tea_block_extent", "tea_cheb_schedule"]
@@ -49,7 +49,8 @@ class Dist(C.Structure):
 class Opts(C.Structure):
     _fields_ = [("presteps", C.c_int), ("eig_margin_lo", C.c_double),
                 ("eig_margin_hi", C.c_double), ("mean_mode", C.c_int), ("loop_mode", C.c_int),
-                ("check_interval", C.c_int), ("profile", C.c_int), ("tile_rows", C.c_int)]
+                ("check_interval", C.c_int), ("profile", C.c_int), ("tile_rows", C.c_int),
+                ("tb_steps", C.c_int), ("tb_rows", C.c_int)]
 
 
 class Stats(C.Structure):
@@ -86,7 +87,7 @@ def lib(build_if_needed: bool = True):
     L.tea_solve.argtypes = [vp, i, d, i, i, C.POINTER(Stats)]
     L.tea_fetch.argtypes = [vp, vp]
     L.tea_set_u.argtypes = [vp, vp]
-    L.tea_kernel_times.argtypes = [vp, vp, vp, i]
+    L.tea_kernel_times.argtypes = [vp, vp, vp, vp, i]
     L.tea_launch_count.argtypes = [vp]
     L.tea_launch_count.restype = C.c_longlong
     L.tea_finalize.argtypes = [vp]
@@ -163,7 +164,8 @@ class Tea:
     def __init__(self, mesh: Mesh, density, energy, dt: float, dist: dict | None = None,
                  presteps: int = 30, eig_margins=(0.95, 1.05), mean_mode: int = 0,
                  loop_mode: int = 0, check_interval: int = 0, profile: bool = False,
-                 tile_rows: int = 0, device=None, stream=None):
+                 tile_rows: int = 0, tb_steps: int = 0, tb_rows: int = 0, device=None,
+                 stream=None):
         import torch
         if not torch.cuda.is_available():
             raise RuntimeError("paper_conf_cluster_mcintosh_smithm17_b200 needs a CUDA device "
@@ -183,7 +185,7 @@ class Tea:
                               dist.get("py", 1), dist.get("halo_depth", 1),
                               C.cast(self._nccl_id, C.c_void_p) if self._nccl_id else None)
         self.opts = Opts(presteps, eig_margins[0], eig_margins[1], mean_mode, loop_mode,
-                         check_interval, 1 if profile else 0, tile_rows)
+                         check_interval, 1 if profile else 0, tile_rows, tb_steps, tb_rows)
         with torch.cuda.device(self.device):
             nbytes = workspace_bytes(mesh, self._dist)
             self.workspace = torch.empty(nbytes, dtype=torch.uint8, device=self.device)
@@ -226,10 +228,12 @@ class Tea:
             raise TeaError(st, self.L.tea_last_error(self.ctx).decode())
 
     def kernel_times(self, reset=False):
+        """{kernel class: (total ms, launches, algorithmic bytes)} in profile mode."""
         ms = (C.c_double * len(KERNELS))()
         n = (C.c_longlong * len(KERNELS))()
-        self.L.tea_kernel_times(self.ctx, ms, n, 1 if reset else 0)
-        return {k: (ms[i], n[i]) for i, k in enumerate(KERNELS)}
+        by = (C.c_double * len(KERNELS))()
+        self.L.tea_kernel_times(self.ctx, ms, n, by, 1 if reset else 0)
+        return {k: (ms[i], n[i], by[i]) for i, k in enumerate(KERNELS)}
 
     def launch_count(self) -> int:
         return int(self.L.tea_launch_count(self.ctx))

@@ -64,7 +64,7 @@ BlockLayout layout_block(const tea_mesh &m, int px, int py, int d, int b) {
     split(m.ny, py, L.bj, &L.gy0, &L.gy1);
     L.bx = L.gx1 - L.gx0;
     L.by = L.gy1 - L.gy0;
-    L.H = d + 2;
+    L.H = std::max(d + 2, kTbMaxSteps + 2);  // the fused passes read M rows past a tile
     L.X0 = (int)round_up(d + 4, 16);
     L.pitch = (int)round_up(L.X0 + L.bx + d + 4, 32);
     L.rows = L.by + 2 * L.H;
@@ -130,6 +130,7 @@ struct tea_ctx {
     size_t evnext = 0;
     double kms[TEA_K_COUNT] = {};
     long long kcount[TEA_K_COUNT] = {};
+    double kbytes[TEA_K_COUNT] = {};
     // graphs: key -> exec
     std::map<long long, cudaGraphExec_t> graphs;
     std::map<long long, int> graph_kernels;
@@ -181,9 +182,10 @@ KArgs kargs(tea_ctx *c, const BlockCtx &b, bool set_cond = false) {
     return a;
 }
 
-// Issue one kernel launch (profiled with an event pair when profiling).
+// Issue one kernel launch (profiled with an event pair when profiling). `bytes` =
+// the launch's algorithmic HBM bytes, accumulated per kernel class.
 template <class F>
-void K(tea_ctx *c, int kid, F &&f) {
+void K(tea_ctx *c, int kid, double bytes, F &&f) {
     if (c->profiling) {
         if (c->evnext + 2 > c->evpool.size()) {
             for (int i = 0; i < 256; ++i) {
@@ -198,6 +200,7 @@ void K(tea_ctx *c, int kid, F &&f) {
         CK(cudaGetLastError());
         CK(cudaEventRecord(b, c->stream));
         c->pending.push_back({kid, a, b});
+        c->kbytes[kid] += bytes;
     } else {
         f();
         CK(cudaGetLastError());
@@ -230,7 +233,7 @@ void reduce(tea_ctx *c, int first, int n) {
     if (nb > 1) {
         std::vector<Scalars *> L;
         for (auto &b : c->blocks) L.push_back(b.S);
-        K(c, TEA_K_SCALAR, [&] { launch_combine(L.data(), nb, n, first, c->stream); });
+        K(c, TEA_K_SCALAR, 0.0, [&] { launch_combine(L.data(), nb, n, first, c->stream); });
     }
     if (c->nranks > 1) {
         double *p = &c->blocks[0].S->red_pw + first;
@@ -249,7 +252,7 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
         if (x.nsend == 0) continue;
         const double *F[4];
         for (int i = 0; i < nf; ++i) F[i] = b.f[fids_per_block_field[i]];
-        K(c, TEA_K_PACK, [&] {
+        K(c, TEA_K_PACK, 0.0, [&] {
             launch_pack(F, nf, b.L.pitch, x.d_send, x.nsend, b.sendbuf, c->stream);
         });
     }
@@ -293,7 +296,7 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
         if (x.nrecv == 0) continue;
         double *F[4];
         for (int i = 0; i < nf; ++i) F[i] = b.f[fids_per_block_field[i]];
-        K(c, TEA_K_UNPACK, [&] {
+        K(c, TEA_K_UNPACK, 0.0, [&] {
             launch_unpack(F, nf, b.L.pitch, x.d_recv, x.nrecv, b.recvbuf, c->stream);
         });
     }
@@ -409,19 +412,26 @@ std::vector<ChebOpS> cheb_schedule(int s, int d) {
             ++i;
             rdep = std::max(rdep, i == 1 ? o.arg + 1 : o.arg);
         }
-    ops[0].arg = std::min(rdep, d);
+    // d >= 2: at least depth 2 so the corners come along (extended regions are
+    // rectangles; their corner cells read r pointwise)
+    ops[0].arg = d > 1 ? std::min(d, std::max(rdep, 2)) : 1;
     (void)step;
     return ops;
 }
 
 // ------------------------------------------------------------------ phase bodies
-int zbuf(int i) { return F_Z0 + ((i - 1) % 3); }  // z_i lives in Z[(i-1)%3]
+int zbuf(int i) { return F_Z0 + ((i - 1) % 3); }  // per-step path: z_i lives in Z[(i-1)%3]
+
+// algorithmic bytes of a launch: streams x 8 B x owned cells
+double sbytes(const BlockCtx &b, int streams) {
+    return 8.0 * streams * (double)b.L.bx * (double)b.L.by;
+}
 
 void body_cg(tea_ctx *c, int par, bool last_sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan(c, R);
-        K(c, TEA_K_SPMV, [&] {
+        K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[F_R0], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
         });
@@ -430,7 +440,7 @@ void body_cg(tea_ctx *c, int par, bool last_sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan(c, R);
-        K(c, TEA_K_UPDATE, [&] {
+        K(c, TEA_K_UPDATE, sbytes(b, 3), [&] {
             launch_update(kargs(c, b, last_sets_cond), L, R, b.f[F_W], b.f[F_R0], c->stream);
         });
     }
@@ -438,14 +448,15 @@ void body_cg(tea_ctx *c, int par, bool last_sets_cond) {
     exchange(c, X_R1, {F_R0});
 }
 
-// Chebyshev chain z = B(A) r. fused: first step also does r_out = r_in - alpha w
-// (single block only). Returns nothing; z_s ends in zbuf(s).
-void cheb_chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond) {
+// Chebyshev chain z = B(A) r, one kernel per step (blocks with neighbours; or
+// tb_steps == 1). fused: the first step also does r_out = r_in - alpha w (single
+// block only). Returns the field holding z_s.
+int cheb_chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond) {
     auto ops = cheb_schedule(s, c->d);
     int r = fused ? rout : rin;
     int step = 0;
     for (auto &op : ops) {
-        if (op.code == 1) {
+        if (op.code == 1) {  // X_RD is depth d >= arg (a superset of what is read)
             if (!fused) exchange(c, op.arg == 1 ? X_R1 : X_RD, {r});
         } else if (op.code == 3) {
             // pair (z_{i-1}, z_{i-2}) before step i = step+1; for i == 2 only z_1 matters
@@ -464,7 +475,8 @@ void cheb_chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, 
                 const double *z1 = step >= 2 ? b.f[zbuf(step - 1)] : nullptr;
                 const double *z2 = step >= 3 ? b.f[zbuf(step - 2)] : nullptr;
                 int kid = step == 1 ? TEA_K_CHEB_FIRST : (last ? TEA_K_CHEB_LAST : TEA_K_CHEB_STEP);
-                K(c, kid, [&] {
+                const int streams = mode == 0 ? (fu ? 6 : 4) : (mode == 1 ? 5 : 6);
+                K(c, kid, sbytes(b, streams), [&] {
                     launch_cheb(kargs(c, b, last && sets_cond), L, R, D, mode, step, last, fu,
                                 restart, b.f[fu ? rin : r], b.f[F_W], b.f[rout], z1, z2,
                                 b.f[zbuf(step)], b.f[F_KX], b.f[F_KY], c->stream);
@@ -473,32 +485,102 @@ void cheb_chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, 
             if (last) reduce(c, 1, 2);
         }
     }
+    return zbuf(s);
+}
+
+// Split s steps into passes of at most Mmax, balanced (e.g. 10 -> 4,3,3).
+std::vector<int> tb_passes(int s, int mmax) {
+    std::vector<int> v;
+    const int P = (s + mmax - 1) / mmax;
+    for (int p = 0; p < P; ++p) v.push_back(s / P + (p < s % P ? 1 : 0));
+    return v;
+}
+
+int tb_steps(const tea_ctx *c) {
+    int m = c->opts.tb_steps;
+    if (m == 0) m = 4;
+    return std::min(m, kTbMaxSteps);
+}
+
+// Temporally blocked chain (single block): passes of M steps, each ONE kernel
+// (tea_cheb_tb.cu). z pairs ping-pong: pass p writes (z_{last-1}, z_last) into
+// pair p%2 = (Z0,Z1) or (Z2,Z3). Returns the field holding z_s.
+int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout,
+                  bool sets_cond) {
+    const auto passes = tb_passes(s, tb_steps(c));
+    const int pairA[2] = {F_Z0, F_Z2}, pairB[2] = {F_Z1, F_Z3};
+    BlockCtx &b = c->blocks[0];
+    const Region R = b.owned();
+    const int jlim = b.L.pitch - b.L.X0;
+    int step0 = 1;
+    const int r = fused ? rout : rin;
+    for (size_t p = 0; p < passes.size(); ++p) {
+        const int M = passes[p];
+        const bool first = p == 0, last = p + 1 == passes.size();
+        const bool fu = fused && first;
+        const int o = p % 2, in = (p + 1) % 2;
+        int ty = c->opts.tb_rows > 0 ? c->opts.tb_rows : 0;
+        if (ty <= 0) {
+            // enough CTAs for ~2 waves of 5 CTAs/SM, tiles tall enough that the
+            // 2M-row pipeline fill stays small
+            ty = 64;
+            while (ty > 16 && tb_ctas(M, R.j1, R.k1, ty) < 1480) ty /= 2;
+        }
+        int streams = first ? (fu ? 4 : 3) : 5;     // reads
+        streams += (fu ? 1 : 0) + (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})
+        const int kid = last ? TEA_K_TB_LAST : (first ? TEA_K_TB_FIRST : TEA_K_TB_MID);
+        K(c, kid, sbytes(b, streams), [&] {
+            launch_cheb_tb(kargs(c, b, last && sets_cond), R, M, ty, jlim, step0, first, fu,
+                           last, restart, b.f[first && fu ? rin : r], b.f[F_W], b.f[rout],
+                           first ? nullptr : b.f[pairB[in]], first ? nullptr : b.f[pairA[in]],
+                           b.f[pairA[o]], b.f[pairB[o]], b.f[F_KX], b.f[F_KY], c->stream);
+        });
+        step0 += M;
+    }
+    reduce(c, 1, 2);
+    return pairB[(passes.size() - 1) % 2];
 }
 
 bool single_block(tea_ctx *c) { return c->px * c->py == 1; }
 
+int chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond) {
+    if (single_block(c) && tb_steps(c) > 1)
+        return cheb_chain_tb(c, s, restart, fused, rin, rout, sets_cond);
+    return cheb_chain(c, s, restart, fused, rin, rout, sets_cond);
+}
+
+// field holding z_s after a chain (same for every chain of a context and s)
+int zs_field(tea_ctx *c, int s) {
+    if (single_block(c) && tb_steps(c) > 1) {
+        const int P = (int)tb_passes(s, tb_steps(c)).size();
+        return (P - 1) % 2 == 0 ? F_Z1 : F_Z3;
+    }
+    return zbuf(s);
+}
+
 void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
     const bool fused = single_block(c);
+    const int zs = zs_field(c, s);
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan(c, R);
-        K(c, TEA_K_SPMV, [&] {
-            launch_spmv(kargs(c, b), L, R, b.f[zbuf(s)], b.f[F_P0 + par], b.f[F_P1 - par],
+        K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
+            launch_spmv(kargs(c, b), L, R, b.f[zs], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
         });
     }
     reduce(c, 0, 1);
     if (fused) {
-        cheb_chain(c, s, false, true, F_R0 + par, F_R1 - par, sets_cond);
+        chain(c, s, false, true, F_R0 + par, F_R1 - par, sets_cond);
     } else {
         for (auto &b : c->blocks) {
             Region R = b.owned();
             Launch L = plan(c, R);
-            K(c, TEA_K_UPDATE, [&] {
+            K(c, TEA_K_UPDATE, sbytes(b, 3), [&] {
                 launch_update_nodot(kargs(c, b), L, R, b.f[F_W], b.f[F_R0], c->stream);
             });
         }
-        cheb_chain(c, s, false, false, F_R0, F_R0, sets_cond);
+        chain(c, s, false, false, F_R0, F_R0, sets_cond);
     }
 }
 
@@ -619,7 +701,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
 
     const int lim1 = method == TEA_CG ? max_iters : std::min(pre, max_iters);
     for (auto &b : c->blocks)
-        K(c, TEA_K_SCALAR, [&] {
+        K(c, TEA_K_SCALAR, 0.0, [&] {
             launch_scalars(kargs(c, b), SC_BEGIN, eps, lim1, max_iters, c->opts.eig_margin_lo,
                            c->opts.eig_margin_hi, c->stream);
         });
@@ -627,14 +709,14 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan(c, R);
-        K(c, TEA_K_RESIDUAL, [&] {
+        K(c, TEA_K_RESIDUAL, sbytes(b, 5), [&] {
             launch_residual(kargs(c, b), L, R, b.f[F_U], b.f[F_KX], b.f[F_KY], b.f[F_U0],
                             b.f[F_R0], c->stream);
         });
     }
     reduce(c, 1, 2);
     for (auto &b : c->blocks)
-        K(c, TEA_K_SCALAR, [&] {
+        K(c, TEA_K_SCALAR, 0.0, [&] {
             launch_scalars(kargs(c, b), SC_R0, 0, 0, 0, 0, 0, c->stream);
         });
     exchange(c, X_R1, {F_R0});
@@ -649,8 +731,8 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
     if (phase2) {
         // ---- eigen-estimate, coefficients, restart z = B(A) r, p = z
         for (auto &b : c->blocks)
-            K(c, TEA_K_EIG, [&] { launch_eig_setup(kargs(c, b), s, c->stream); });
-        cheb_chain(c, s, true, false, F_R0, F_R0, false);
+            K(c, TEA_K_EIG, 0.0, [&] { launch_eig_setup(kargs(c, b), s, c->stream); });
+        chain(c, s, true, false, F_R0, F_R0, false);
         read_state(c);
         if (!c->hS->done) {
             long long key = 2 + 16LL * s;
@@ -858,7 +940,7 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
             Region all{-d, L.bx + d + 1, -d, L.by + d + 1};
             Region kxr{-d, L.bx + d + 1, -d, L.by + d};
             Region kyr{-d, L.bx + d, -d, L.by + d + 1};
-            K(c.get(), TEA_K_INIT, [&] {
+            K(c.get(), TEA_K_INIT, 0.0, [&] {
                 launch_init_fields(kargs(c.get(), b), b.f[F_W], b.f[F_Z0], b.f[F_U0], b.f[F_U],
                                    b.f[F_KX], b.f[F_KY], owned, all, kxr, kyr, c->rx, c->ry,
                                    o.mean_mode, c->stream);
@@ -929,15 +1011,18 @@ tea_status tea_set_u(tea_ctx *ctx, const double *u_host) {
     }
 }
 
-tea_status tea_kernel_times(tea_ctx *ctx, double *ms, long long *launches, int reset) {
+tea_status tea_kernel_times(tea_ctx *ctx, double *ms, long long *launches, double *bytes,
+                            int reset) {
     if (!ctx) return TEA_ERR_ARG;
     for (int i = 0; i < TEA_K_COUNT; ++i) {
         if (ms) ms[i] = ctx->kms[i];
         if (launches) launches[i] = ctx->kcount[i];
+        if (bytes) bytes[i] = ctx->kbytes[i];
     }
     if (reset) {
         std::memset(ctx->kms, 0, sizeof ctx->kms);
         std::memset(ctx->kcount, 0, sizeof ctx->kcount);
+        std::memset(ctx->kbytes, 0, sizeof ctx->kbytes);
     }
     return TEA_OK;
 }

@@ -56,7 +56,7 @@ struct Region {
 
 // Field indices inside a block's workspace.
 enum Field {
-    F_U0 = 0, F_U, F_KX, F_KY, F_R0, F_R1, F_P0, F_P1, F_W, F_Z0, F_Z1, F_Z2, F_COUNT
+    F_U0 = 0, F_U, F_KX, F_KY, F_R0, F_R1, F_P0, F_P1, F_W, F_Z0, F_Z1, F_Z2, F_Z3, F_COUNT
 };
 
 // Launch geometry of one stencil / pointwise launch.
@@ -114,5 +114,15 @@ void launch_unpack(double *const *fields, int nf, int pitch, const int *boxes, i
                    const double *buf, cudaStream_t st);
 
 enum { SC_BEGIN = 0, SC_R0 = 1, SC_PHASE2 = 2 };
+
+// Temporally blocked Chebyshev passes (tea_cheb_tb.cu).
+constexpr int kTbMaxSteps = 5;
+int tb_out_cols(int M);
+int tb_ctas(int M, int width, int height, int ty);
+void launch_cheb_tb(const KArgs &a, const Region &R, int M, int ty, int jlim, int step0,
+                    bool first, bool fuse, bool last, bool restart, const double *rin,
+                    const double *win, double *rout, const double *zin1, const double *zin2,
+                    double *zoutA, double *zoutB, const double *kx, const double *ky,
+                    cudaStream_t st);
 
 }  // namespace tea

@@ -248,3 +248,42 @@ def test_multiblock_fixed_iterations(tea, ora, px, py, d):
                             method=method, eps=0.0, max_iters=k, inner_steps=6)
         assert st_g[0]["iterations"] == k
         assert field_err(u_g, u_o, "random") <= 1e-12
+
+
+# ---------------------------------------------------------------- fused passes
+# Temporally blocked Chebyshev passes (tea_cheb_tb.cu, on-chip matrix powers): M steps
+# per kernel; tb_steps = 1 is the one-kernel-per-step path.
+@pytest.mark.parametrize("tb", [1, 2, 3, 4, 5])
+@pytest.mark.parametrize("s", [1, 2, 3, 5, 10, 13])
+def test_fused_passes_converged(tea, ora, tb, s):
+    deck = deck_of("pipe", 256, 200)
+    kw = dict(method=1, eps=1e-13, max_iters=20000, inner_steps=s)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, tb_steps=tb, **kw)
+    assert st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+
+
+@pytest.mark.parametrize("kind,nx,ny", [("random", 300, 200), ("random", 257, 65),
+                                        ("random", 1, 97), ("random", 95, 1),
+                                        ("random", 3, 5), ("pipe", 128, 128)])
+@pytest.mark.parametrize("tb", [2, 4, 5])
+def test_fused_passes_fixed_iterations(tea, ora, kind, nx, ny, tb):
+    """30 presteps + 3 outer iterations, eps = 0: agreement to rounding on ragged shapes."""
+    deck = deck_of(kind, nx, ny, seed=4, dt=0.04)
+    kw = dict(method=1, eps=0.0, max_iters=33, inner_steps=7)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, tb_steps=tb, **kw)
+    assert st_g[0]["iterations"] == st_o[0]["iterations"]
+    assert field_err(u_g, u_o, kind) <= 1e-12
+
+
+@pytest.mark.parametrize("tb_rows", [16, 32, 64, 128])
+def test_fused_pass_tile_heights(tea, ora, tb_rows):
+    deck = deck_of("pipe", 384, 300)
+    kw = dict(method=1, eps=1e-12, max_iters=20000, inner_steps=10)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, tb_steps=4, tb_rows=tb_rows, **kw)
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
