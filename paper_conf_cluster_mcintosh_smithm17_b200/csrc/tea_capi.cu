@@ -498,7 +498,13 @@ std::vector<int> tb_passes(int s, int mmax) {
 
 int tb_steps(const tea_ctx *c) {
     int m = c->opts.tb_steps;
-    if (m == 0) m = 4;
+    if (m == 0) {
+        // measured (profiles/r01_tb_sweep.txt): fusing pays once the working set
+        // (13 fields) leaves L2 -- 4096^2: 5 steps/pass 755 us vs 1520 us per outer;
+        // at 1024^2 (L2-resident) one kernel per step is faster (86 vs 87-100 us).
+        const double cells = (double)c->blocks[0].L.bx * c->blocks[0].L.by;
+        m = cells >= 2.0e6 ? kTbMaxSteps : 1;
+    }
     return std::min(m, kTbMaxSteps);
 }
 
