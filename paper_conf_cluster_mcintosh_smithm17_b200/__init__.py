@@ -72,11 +72,14 @@ def lib(build_if_needed: bool = True):
     global _lib
     if _lib is not None:
         return _lib
-    if build_if_needed and _build.stale():
-        _build.build()
-    if not os.path.exists(_build.LIB):
-        raise ImportError(f"CUDA library {_build.LIB} is missing; run __graft_entry__.build()")
-    L = C.CDLL(_build.LIB)
+    path = os.environ.get("TEA_B200_LIB")  # experiments: an alternative build of the same ABI
+    if path is None:
+        if build_if_needed and _build.stale():
+            _build.build()
+        path = _build.LIB
+    if not os.path.exists(path):
+        raise ImportError(f"CUDA library {path} is missing; run __graft_entry__.build()")
+    L = C.CDLL(path)
     vp, i, d = C.c_void_p, C.c_int, C.c_double
     L.tea_version.restype = C.c_char_p
     L.tea_abi_version.restype = i

@@ -530,7 +530,7 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
             // enough CTAs for ~2 waves of 5 CTAs/SM, tiles tall enough that the
             // 2M-row pipeline fill stays small
             ty = 64;
-            while (ty > 16 && tb_ctas(M, R.j1, R.k1, ty) < 1480) ty /= 2;
+            while (ty > 16 && tb_ctas(M, R.j1, R.k1, ty) < 888) ty /= 2;
         }
         int streams = first ? (fu ? 4 : 3) : 5;     // reads
         streams += (fu ? 1 : 0) + (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})

@@ -106,6 +106,12 @@ __device__ bool grid_arrive2(unsigned *ticket) {
 
 }  // namespace
 
+#ifndef TEA_TB_UNROLL
+#define TEA_TB_UNROLL 1
+#endif
+constexpr int kTbUnroll = TEA_TB_UNROLL;  // measured: 2 (step t+1 of row k overlapping
+                                          // step t of row k+1) costs registers, no gain
+
 template <int M>
 struct TbGeom {
     static constexpr int MR = (M + 1) & ~1;  // margin, even (double2 alignment)
@@ -113,8 +119,11 @@ struct TbGeom {
     static constexpr int D = M + 2;             // delay-line depth (rows)
 };
 
+#ifndef TEA_TB_MINB
+#define TEA_TB_MINB 1
+#endif
 template <int M, bool FIRST, bool FUSE, bool LAST>
-__global__ void __launch_bounds__(kThreads)
+__global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
     k_cheb_tb(const double *__restrict__ rin, const double *__restrict__ win,
               double *__restrict__ rout, const double *__restrict__ zin1,
               const double *__restrict__ zin2, double *__restrict__ zoutA,
@@ -200,6 +209,7 @@ __global__ void __launch_bounds__(kThreads)
     };
     const int kbeg = kt0 - M, kend = kt1 + M;
     load(kbeg);
+#pragma unroll(kTbUnroll)
     for (int k = kbeg; k < kend; ++k) {
         double2 X = pX, Wv = pW, Z2 = pZ2, KX = pKx, KY = pKy, RR = pR;
         if (k + 1 < kend) load(k + 1);
