@@ -885,6 +885,9 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
             if (o.eig_margin_hi == 0.0) o.eig_margin_hi = 1.05;
         }
         if (o.loop_mode < 0 || o.loop_mode > 2) fail(TEA_ERR_ARG, "bad loop_mode");
+        // NCCL kernels inside a WHILE-conditional graph body are not a supported
+        // capture target: multi-process runs use chunked graphs (same kernels).
+        if (nranks > 1 && o.loop_mode == 0) o.loop_mode = 1;
         c->opts = o;
         for (long long i = 0; i < (long long)mesh->nx * mesh->ny; i += 1 + ((long long)mesh->nx * mesh->ny) / 4096)
             if (!(density[i] > 0.0)) fail(TEA_ERR_ARG, "density must be > 0");
