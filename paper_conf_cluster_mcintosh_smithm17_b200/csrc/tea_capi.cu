@@ -527,10 +527,14 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
         const int o = p % 2, in = (p + 1) % 2;
         int ty = c->opts.tb_rows > 0 ? c->opts.tb_rows : 0;
         if (ty <= 0) {
-            // enough CTAs for ~2 waves of 5 CTAs/SM, tiles tall enough that the
-            // 2M-row pipeline fill stays small
-            ty = 64;
-            while (ty > 16 && tb_ctas(M, R.j1, R.k1, ty) < 888) ty /= 2;
+            // tall tiles keep the 2M-row pipeline fill small; enough CTAs for ~2 waves
+            // at 3 CTAs/SM. Measured at 4096^2, M = 5 (profiles/r01_tb_rows.txt):
+            // 96 rows 667 us/outer, 64 rows 688, 32 rows 754.
+            const int cand[] = {96, 64, 32, 16};
+            for (int cnd : cand) {
+                ty = cnd;
+                if (tb_ctas(M, R.j1, R.k1, ty) >= 800) break;
+            }
         }
         int streams = first ? (fu ? 4 : 3) : 5;     // reads
         streams += (fu ? 1 : 0) + (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})
