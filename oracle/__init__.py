@@ -26,7 +26,7 @@ _SRC = os.path.join(_HERE, "tea_oracle.c")
 _LIB = os.path.join(_HERE, "libtea_oracle.so")
 CFLAGS = ["-O2", "-ffp-contract=off", "-fno-fast-math", "-std=c99", "-fPIC", "-shared"]
 
-CG, CPPCG = 0, 1
+CG, CPPCG, BJCG = 0, 1, 2
 OK, NOT_CONVERGED, ERR_ARG, ERR_BREAKDOWN = 0, 1, -1, -4
 PRESTEPS = 30  # reading R6
 
@@ -72,6 +72,10 @@ def lib():
         L.ora_cheb_coeffs.argtypes = [d, d, i, C.POINTER(d), dp, dp]
         L.ora_cheb_apply.argtypes = [i, i, dp, dp, i, d, dp, dp, dp, dp, dp, dp, dp]
         L.ora_solve.argtypes = [i, i, dp, dp, dp, dp, i, d, i, i, i, C.POINTER(OraStats)]
+        ip = np.ctypeslib.ndpointer(dtype=np.int32, flags="C_CONTIGUOUS")
+        L.ora_solve_ex.argtypes = [i, i, dp, dp, dp, dp, i, d, i, i, i, i, ip,
+                                   C.POINTER(OraStats)]
+        L.ora_bj_apply.argtypes = [i, i, dp, dp, i, ip, dp, dp]
         L.ora_timestep.argtypes = [i, i, d, d, d, d, dp, dp, d, i, d, i, i, i, i, dp,
                                    C.POINTER(OraStats)]
         _lib = L
@@ -153,6 +157,15 @@ def cheb_apply(Kx, Ky, s, theta, a, b, r):
     return z
 
 
+def bj_apply(Kx, Ky, r, ybounds=None):
+    """z = M^{-1} r, M = block-Jacobi strips of 4 along y (reading R18)."""
+    ny, nx = r.shape
+    yb = np.ascontiguousarray([0, ny] if ybounds is None else ybounds, dtype=np.int32)
+    z = np.zeros((ny, nx))
+    lib().ora_bj_apply(nx, ny, _c(Kx), _c(Ky), yb.size - 1, yb, _c(r), z)
+    return z
+
+
 @dataclass
 class Result:
     u: np.ndarray
@@ -161,13 +174,15 @@ class Result:
 
 
 def solve(Kx, Ky, u0, u_init=None, method=CG, eps=1e-10, max_iters=10000, inner_steps=10,
-          presteps=PRESTEPS):
-    """One linear solve A u = u0 from initial guess u_init (default u0)."""
+          presteps=PRESTEPS, ybounds=None):
+    """One linear solve A u = u0 from initial guess u_init (default u0). ybounds: the
+    block-row boundaries that truncate the block-Jacobi strips (default one block)."""
     ny, nx = u0.shape
     u = _c(u0 if u_init is None else u_init).copy()
     st = OraStats()
-    s = lib().ora_solve(nx, ny, _c(Kx), _c(Ky), _c(u0), u, method, eps, max_iters,
-                        inner_steps, presteps, C.byref(st))
+    yb = np.ascontiguousarray([0, ny] if ybounds is None else ybounds, dtype=np.int32)
+    s = lib().ora_solve_ex(nx, ny, _c(Kx), _c(Ky), _c(u0), u, method, eps, max_iters,
+                           inner_steps, presteps, yb.size - 1, yb, C.byref(st))
     return Result(u, s, st.as_dict())
 
 
@@ -183,7 +198,7 @@ def timestep(deck, method=CG, eps=1e-10, max_iters=10000, inner_steps=10,
 
 
 def run(deck, steps=1, method=CG, eps=1e-10, max_iters=10000, inner_steps=10,
-        presteps=PRESTEPS, mean_mode=0):
+        presteps=PRESTEPS, mean_mode=0, ybounds=None):
     """`steps` implicit timesteps: u^{n+1} = A^{-1} u^n, u^0 = rho*e (reading R4).
 
     Returns (u, [stats per step], [status per step]).
@@ -193,7 +208,7 @@ def run(deck, steps=1, method=CG, eps=1e-10, max_iters=10000, inner_steps=10,
     u = _c(deck.density) * _c(deck.energy)  # reading R4 (TeaLeaf): u = rho * e
     stats, statuses = [], []
     for _ in range(steps):
-        res = solve(Kx, Ky, u, None, method, eps, max_iters, inner_steps, presteps)
+        res = solve(Kx, Ky, u, None, method, eps, max_iters, inner_steps, presteps, ybounds)
         u = res.u
         stats.append(res.stats)
         statuses.append(res.status)
