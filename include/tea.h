@@ -43,7 +43,11 @@ typedef enum {
     TEA_ERR_STATE = -5      /* call out of order / context already failed             */
 } tea_status;
 
-typedef enum { TEA_CG = 0, TEA_CPPCG = 1 } tea_method;
+/* TEA_BJCG: CG preconditioned by block Jacobi on 4-cell strips along y, each a
+ * tridiagonal block of A solved by the Thomas algorithm, strips truncated at the mesh
+ * edge and at block boundaries (Sec. IV.C.1). Halo depth 1:
+ * block Jacobi does not combine with matrix powers.                    */
+typedef enum { TEA_CG = 0, TEA_CPPCG = 1, TEA_BJCG = 2 } tea_method;
 
 typedef struct tea_ctx tea_ctx; /* opaque, library-owned */
 
@@ -106,6 +110,7 @@ enum {
     TEA_K_INIT = 0, TEA_K_RESIDUAL, TEA_K_SPMV, TEA_K_UPDATE, TEA_K_CHEB_FIRST,
     TEA_K_CHEB_STEP, TEA_K_CHEB_LAST, TEA_K_EIG, TEA_K_PACK, TEA_K_UNPACK, TEA_K_SCALAR,
     TEA_K_TB_FIRST, TEA_K_TB_MID, TEA_K_TB_LAST, /* fused multi-step Chebyshev passes */
+    TEA_K_BJ,                                     /* block-Jacobi update + strip solves  */
     TEA_K_COUNT
 };
 

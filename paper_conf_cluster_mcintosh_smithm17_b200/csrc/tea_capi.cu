@@ -594,6 +594,28 @@ void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
     }
 }
 
+// Block-Jacobi PCG outer iteration (Sec. IV.C.1): spmv on z; fused update + strip solves.
+void body_bj(tea_ctx *c, int par, bool sets_cond) {
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan(c, R);
+        K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
+            launch_spmv(kargs(c, b), L, R, b.f[F_Z0], b.f[F_P0 + par], b.f[F_P1 - par],
+                        b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
+        });
+    }
+    reduce(c, 0, 1);
+    for (auto &b : c->blocks) {
+        // reads r, w, Ky, c', 1/den; writes r, z
+        K(c, TEA_K_BJ, sbytes(b, 7), [&] {
+            launch_bj(kargs(c, b), b.owned(), true, sets_cond, b.f[F_W], b.f[F_R0], b.f[F_Z0],
+                      b.f[F_KY], b.f[F_BJC], b.f[F_BJD], c->stream);
+        });
+    }
+    reduce(c, 1, 2);
+    exchange(c, X_Z1, {F_Z0});
+}
+
 void read_state(tea_ctx *c) {
     CK(cudaMemcpyAsync(c->hS, c->blocks[0].S, offsetof(Scalars, cheb_a),
                        cudaMemcpyDeviceToHost, c->stream));
@@ -696,7 +718,8 @@ tea_status map_status(int ds, bool maxed) {
 tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, int s,
                       tea_stats *st) {
     if (c->failed) fail(TEA_ERR_STATE, "context already failed: %s", c->err.c_str());
-    if (method != TEA_CG && method != TEA_CPPCG) fail(TEA_ERR_ARG, "bad method %d", (int)method);
+    if (method != TEA_CG && method != TEA_CPPCG && method != TEA_BJCG)
+        fail(TEA_ERR_ARG, "bad method %d", (int)method);
     if (max_iters < 0) fail(TEA_ERR_ARG, "max_iters < 0");
     if (method == TEA_CPPCG && (s < 1 || s > kMaxS))
         fail(TEA_ERR_ARG, "inner_steps must be in [1,%d]", kMaxS);
@@ -709,7 +732,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
     CK(cudaStreamWaitEvent(c->stream, c->ev_in, 0));
     CK(cudaEventRecord(c->ev_t0, c->stream));
 
-    const int lim1 = method == TEA_CG ? max_iters : std::min(pre, max_iters);
+    const int lim1 = method == TEA_CPPCG ? std::min(pre, max_iters) : max_iters;
     for (auto &b : c->blocks)
         K(c, TEA_K_SCALAR, 0.0, [&] {
             launch_scalars(kargs(c, b), SC_BEGIN, eps, lim1, max_iters, c->opts.eig_margin_lo,
@@ -725,16 +748,30 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         });
     }
     reduce(c, 1, 2);
+    if (method == TEA_BJCG) {  // z = M^{-1} r, r.z, r.r (no update)
+        for (auto &b : c->blocks)
+            K(c, TEA_K_BJ, sbytes(b, 5), [&] {
+                launch_bj(kargs(c, b), b.owned(), false, false, b.f[F_W], b.f[F_R0], b.f[F_Z0],
+                          b.f[F_KY], b.f[F_BJC], b.f[F_BJD], c->stream);
+            });
+        reduce(c, 1, 2);
+    }
     for (auto &b : c->blocks)
         K(c, TEA_K_SCALAR, 0.0, [&] {
             launch_scalars(kargs(c, b), SC_R0, 0, 0, 0, 0, 0, c->stream);
         });
-    exchange(c, X_R1, {F_R0});
+    if (method == TEA_BJCG)
+        exchange(c, X_Z1, {F_Z0});
+    else
+        exchange(c, X_R1, {F_R0});
     read_state(c);
 
-    // ---- phase 1: CG (or the CPPCG presteps)
+    // ---- phase 1: CG (or the CPPCG presteps), or block-Jacobi PCG
     if (!c->hS->done) {
-        run_loop(c, 1, lim1, [&](int par, bool sc) { body_cg(c, par, sc); });
+        if (method == TEA_BJCG)
+            run_loop(c, 3, lim1, [&](int par, bool sc) { body_bj(c, par, sc); });
+        else
+            run_loop(c, 1, lim1, [&](int par, bool sc) { body_cg(c, par, sc); });
     }
     int ds = c->hS->status;
     bool phase2 = method == TEA_CPPCG && ds == DS_LIMIT && c->hS->it < max_iters;
@@ -957,6 +994,10 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
                 launch_init_fields(kargs(c.get(), b), b.f[F_W], b.f[F_Z0], b.f[F_U0], b.f[F_U],
                                    b.f[F_KX], b.f[F_KY], owned, all, kxr, kyr, c->rx, c->ry,
                                    o.mean_mode, c->stream);
+            });
+            K(c.get(), TEA_K_INIT, 0.0, [&] {
+                launch_bj_setup(kargs(c.get(), b), owned, b.f[F_KX], b.f[F_KY], b.f[F_BJC],
+                                b.f[F_BJD], c->stream);
             });
             // the staging fields are solver fields with zero halos: clear them again
             CK(cudaMemsetAsync(ws + F_W * L.field_bytes, 0, L.field_bytes, c->stream));

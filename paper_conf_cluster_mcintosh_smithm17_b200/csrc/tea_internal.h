@@ -56,7 +56,9 @@ struct Region {
 
 // Field indices inside a block's workspace.
 enum Field {
-    F_U0 = 0, F_U, F_KX, F_KY, F_R0, F_R1, F_P0, F_P1, F_W, F_Z0, F_Z1, F_Z2, F_Z3, F_COUNT
+    F_U0 = 0, F_U, F_KX, F_KY, F_R0, F_R1, F_P0, F_P1, F_W, F_Z0, F_Z1, F_Z2, F_Z3,
+    F_BJC, F_BJD,  // block-Jacobi Thomas coefficients c'_i and 1/den_i
+    F_COUNT
 };
 
 // Launch geometry of one stencil / pointwise launch.
@@ -114,6 +116,14 @@ void launch_unpack(double *const *fields, int nf, int pitch, const int *boxes, i
                    const double *buf, cudaStream_t st);
 
 enum { SC_BEGIN = 0, SC_R0 = 1, SC_PHASE2 = 2 };
+
+// Block-Jacobi (tea_kernels.cu): Thomas coefficients once; per iteration
+// r -= alpha w (update) then z = M^{-1} r on 4-row strips, r.z and r.r.
+void launch_bj_setup(const KArgs &a, const Region &R, const double *kx, const double *ky,
+                     double *bjc, double *bjd, cudaStream_t st);
+void launch_bj(const KArgs &a, const Region &R, bool update, bool sets_cond, const double *w,
+               double *r, double *z, const double *ky, const double *bjc, const double *bjd,
+               cudaStream_t st);
 
 // Temporally blocked Chebyshev passes (tea_cheb_tb.cu).
 constexpr int kTbMaxSteps = 5;

@@ -302,3 +302,46 @@ def test_fused_pass_tile_heights(tea, ora, tb_rows):
     u_g, st_g = gpu_run(tea, deck, tb_steps=4, tb_rows=tb_rows, **kw)
     assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
     assert rel_err(u_g, u_o) <= 1e-10
+
+
+# ---------------------------------------------------------------- block Jacobi (NEXT-1)
+def ybounds_of(tea, deck, px, py):
+    m = tea.mesh_of(deck)
+    return [tea.block_extent(m, px, py, bj * px)[2] for bj in range(py)] + [deck.ny]
+
+
+@pytest.mark.parametrize("kind,nx,ny", [("pipe", 128, 128), ("pipe", 256, 200),
+                                        ("random", 300, 203), ("random", 257, 65),
+                                        ("random", 1, 97), ("random", 95, 1), ("random", 3, 5)])
+def test_bjcg_converged(tea, ora, kind, nx, ny):
+    deck = deck_of(kind, nx, ny, seed=6)
+    kw = dict(method=2, eps=1e-13, max_iters=20000)
+    u_o, st_o, s_o = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, **kw)
+    assert s_o[0] == 0 and st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert field_err(u_g, u_o, kind) <= 1e-10
+
+
+@pytest.mark.parametrize("kind,nx,ny,k", [("random", 300, 203, 5), ("pipe", 130, 97, 12),
+                                          ("random", 64, 7, 3)])
+def test_bjcg_fixed_iterations(tea, ora, kind, nx, ny, k):
+    deck = deck_of(kind, nx, ny, seed=8, dt=0.04)
+    kw = dict(method=2, eps=0.0, max_iters=k)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, **kw)
+    assert st_g[0]["iterations"] == k
+    assert field_err(u_g, u_o, kind) <= 1e-12
+
+
+@pytest.mark.parametrize("px,py", [(2, 1), (1, 3), (3, 2), (2, 4)])
+def test_bjcg_multiblock(tea, ora, px, py):
+    """Strips are truncated at block-row boundaries: the oracle gets the
+    same boundaries (ybounds)."""
+    deck = deck_of("pipe", 200, 170)
+    yb = ybounds_of(tea, deck, px, py)
+    kw = dict(method=2, eps=1e-13, max_iters=20000)
+    u_o, st_o, _ = ora.run(deck, steps=1, ybounds=yb, **kw)
+    u_g, st_g = gpu_run(tea, deck, dist=dict(px=px, py=py, halo_depth=1, nranks=1), **kw)
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
