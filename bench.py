@@ -142,7 +142,7 @@ def run_reference(args):
         return 0
     oracle.build()
     deck = inputs.crooked_pipe(args.n)
-    method = oracle.CPPCG if args.method == "cppcg" else oracle.CG
+    method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG}[args.method]
     sample_iters = args.ref_iters
     for _ in range(args.warmup):  # untimed warm-up (page-in, caches)
         oracle.run(deck, steps=1, method=method, eps=args.eps, max_iters=1,
@@ -156,9 +156,9 @@ def run_reference(args):
         its += st[0]["iterations"]
         mv += st[0]["matvecs"]
     value = its / t_all
-    sample = (f"first {sample_iters} iterations of timestep 1 "
-              f"({'30 CG presteps + ' + str(sample_iters - 30) + ' CPPCG outer' if method else 'CG'})"
-              f" per step, serial C oracle")
+    sample = (f"first {sample_iters} iterations of timestep 1 ("
+              + (f"30 CG presteps + {sample_iters - 30} CPPCG outer" if args.method == "cppcg"
+                 else METHOD_NAME[args.method]) + ") per step, serial C oracle")
     line = {
         "impl": "reference", "metric": metric_name(args), "value": value, "unit": "iterations/s",
         "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
@@ -174,14 +174,17 @@ def run_reference(args):
     return 0
 
 
+METHOD_NAME = {"cppcg": "CPPCG", "cg": "CG", "bjcg": "block-Jacobi PCG"}
+
+
 def metric_name(args):
-    return (f"solver iterations/s, {args.n}^2 {'CPPCG' if args.method == 'cppcg' else 'CG'}"
+    return (f"solver iterations/s, {args.n}^2 {METHOD_NAME[args.method]}"
             f" (time-to-solution, HBM GB/s alongside)")
 
 
 def config(args):
     return {"workload": f"crooked_pipe {args.n}x{args.n} "
-                        f"{'CPPCG s=' + str(args.inner) if args.method == 'cppcg' else 'CG'}"
+                        f"{'CPPCG s=' + str(args.inner) if args.method == 'cppcg' else METHOD_NAME[args.method]}"
                         f" eps={args.eps:g} 1 timestep/step",
             "mesh": [args.n, args.n], "method": args.method, "inner_steps": args.inner,
             "eps": args.eps, "halo_depth": args.halo_depth, "dt": 0.004,
@@ -193,16 +196,17 @@ def config(args):
 def cpu_baseline(args, deck):
     import oracle
     oracle.build()
-    method = oracle.CPPCG if args.method == "cppcg" else oracle.CG
+    method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG}[args.method]
     t0 = time.perf_counter()
     _, st, _ = oracle.run(deck, steps=1, method=method, eps=args.eps, max_iters=args.ref_iters,
                           inner_steps=args.inner)
     dt = time.perf_counter() - t0
     return {"value": st[0]["iterations"] / dt, "unit": "iterations/s", "cores": 1,
             "kind": "oracle",
-            "sample": f"first {args.ref_iters} iterations of timestep 1 "
-                      f"({st[0]['presteps'] or st[0]['iterations']} CG + {st[0]['outer']} CPPCG"
-                      f" outer), serial C oracle, {dt:.1f} s",
+            "sample": f"first {args.ref_iters} iterations of timestep 1 ("
+                      + (f"{st[0]['presteps']} CG presteps + {st[0]['outer']} CPPCG outer"
+                         if args.method == "cppcg" else METHOD_NAME[args.method])
+                      + f"), serial C oracle, {dt:.1f} s",
             "matvecs_per_s": st[0]["matvecs"] / dt}
 
 
@@ -256,7 +260,7 @@ def run_gpu(args):
         return float(t.item())
 
     deck = inputs.crooked_pipe(args.n)
-    method = tea.CPPCG if args.method == "cppcg" else tea.CG
+    method = {"cppcg": tea.CPPCG, "cg": tea.CG, "bjcg": tea.BJCG}[args.method]
     cells = args.n * args.n
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
                 tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode)
@@ -290,6 +294,8 @@ def run_gpu(args):
         model_bytes = sum(5 * 8 * cells + s["presteps"] * cg_iter_bytes(cells) +
                           outer_bytes(cells, args.inner) - 10 * 8 * cells +  # restart chain
                           s["outer"] * outer_bytes(cells, args.inner) for s in stats)
+    elif method == tea.BJCG:
+        model_bytes = len(stats) * 10 * 8 * cells + iters * 15 * 8 * cells
     else:
         model_bytes = len(stats) * 5 * 8 * cells + iters * cg_iter_bytes(cells)
 
@@ -375,7 +381,7 @@ def main():
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", default="b200", choices=["b200", "reference"])
     ap.add_argument("--n", type=int, default=4096)
-    ap.add_argument("--method", default="cppcg", choices=["cppcg", "cg"])
+    ap.add_argument("--method", default="cppcg", choices=["cppcg", "cg", "bjcg"])
     ap.add_argument("--inner", type=int, default=10)
     ap.add_argument("--eps", type=float, default=1e-12)
     ap.add_argument("--max-iters", type=int, default=100000)
