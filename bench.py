@@ -142,7 +142,8 @@ def run_reference(args):
         return 0
     oracle.build()
     deck = inputs.crooked_pipe(args.n)
-    method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG}[args.method]
+    method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
+              "cg1": oracle.CG1}[args.method]
     sample_iters = args.ref_iters
     for _ in range(args.warmup):  # untimed warm-up (page-in, caches)
         oracle.run(deck, steps=1, method=method, eps=args.eps, max_iters=1,
@@ -174,7 +175,8 @@ def run_reference(args):
     return 0
 
 
-METHOD_NAME = {"cppcg": "CPPCG", "cg": "CG", "bjcg": "block-Jacobi PCG"}
+METHOD_NAME = {"cppcg": "CPPCG", "cg": "CG", "bjcg": "block-Jacobi PCG",
+               "cg1": "single-reduction CG"}
 
 
 def metric_name(args):
@@ -196,7 +198,8 @@ def config(args):
 def cpu_baseline(args, deck):
     import oracle
     oracle.build()
-    method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG}[args.method]
+    method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
+              "cg1": oracle.CG1}[args.method]
     t0 = time.perf_counter()
     _, st, _ = oracle.run(deck, steps=1, method=method, eps=args.eps, max_iters=args.ref_iters,
                           inner_steps=args.inner)
@@ -260,7 +263,8 @@ def run_gpu(args):
         return float(t.item())
 
     deck = inputs.crooked_pipe(args.n)
-    method = {"cppcg": tea.CPPCG, "cg": tea.CG, "bjcg": tea.BJCG}[args.method]
+    method = {"cppcg": tea.CPPCG, "cg": tea.CG, "bjcg": tea.BJCG,
+              "cg1": tea.CG1}[args.method]
     cells = args.n * args.n
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
                 tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode)
@@ -294,6 +298,8 @@ def run_gpu(args):
         model_bytes = sum(5 * 8 * cells + s["presteps"] * cg_iter_bytes(cells) +
                           outer_bytes(cells, args.inner) - 10 * 8 * cells +  # restart chain
                           s["outer"] * outer_bytes(cells, args.inner) for s in stats)
+    elif method == tea.CG1:
+        model_bytes = len(stats) * 9 * 8 * cells + iters * 12 * 8 * cells
     elif method == tea.BJCG:
         model_bytes = len(stats) * 10 * 8 * cells + iters * 15 * 8 * cells
     else:
@@ -381,7 +387,7 @@ def main():
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", default="b200", choices=["b200", "reference"])
     ap.add_argument("--n", type=int, default=4096)
-    ap.add_argument("--method", default="cppcg", choices=["cppcg", "cg", "bjcg"])
+    ap.add_argument("--method", default="cppcg", choices=["cppcg", "cg", "bjcg", "cg1"])
     ap.add_argument("--inner", type=int, default=10)
     ap.add_argument("--eps", type=float, default=1e-12)
     ap.add_argument("--max-iters", type=int, default=100000)

@@ -47,7 +47,11 @@ typedef enum {
  * tridiagonal block of A solved by the Thomas algorithm, strips truncated at the mesh
  * edge and at block boundaries (Sec. IV.C.1). Halo depth 1:
  * block Jacobi does not combine with matrix powers.                    */
-typedef enum { TEA_CG = 0, TEA_CPPCG = 1, TEA_BJCG = 2 } tea_method;
+/* TEA_CG1: single-reduction CG (Chronopoulos & Gear): r.r and (A r).r in ONE global
+ * reduction per iteration, s = A p carried by recurrence -- the restructuring the
+ * paper names as future work. Same iterates as CG in
+ * exact arithmetic; one fused kernel per iteration on a single block.             */
+typedef enum { TEA_CG = 0, TEA_CPPCG = 1, TEA_BJCG = 2, TEA_CG1 = 3 } tea_method;
 
 typedef struct tea_ctx tea_ctx; /* opaque, library-owned */
 
@@ -111,6 +115,7 @@ enum {
     TEA_K_CHEB_STEP, TEA_K_CHEB_LAST, TEA_K_EIG, TEA_K_PACK, TEA_K_UNPACK, TEA_K_SCALAR,
     TEA_K_TB_FIRST, TEA_K_TB_MID, TEA_K_TB_LAST, /* fused multi-step Chebyshev passes */
     TEA_K_BJ,                                     /* block-Jacobi update + strip solves  */
+    TEA_K_CG1, TEA_K_CG1W,                        /* single-reduction CG: fused / A r    */
     TEA_K_COUNT
 };
 

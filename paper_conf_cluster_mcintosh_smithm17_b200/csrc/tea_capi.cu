@@ -616,6 +616,41 @@ void body_bj(tea_ctx *c, int par, bool sets_cond) {
     exchange(c, X_Z1, {F_Z0});
 }
 
+// Single-reduction CG iteration (Chronopoulos-Gear): one fused kernel on a
+// single block (r, w, s ping-pong: Z0/Z1 hold w, Z2/Z3 hold s); update -> halo -> A r
+// with blocks. Either way ONE reduction [del, gam, rr] per iteration.
+void body_cg1(tea_ctx *c, int par, bool sets_cond) {
+    if (single_block(c)) {
+        BlockCtx &b = c->blocks[0];
+        Region R = b.owned();
+        Launch L = plan(c, R);
+        K(c, TEA_K_CG1, sbytes(b, 12), [&] {
+            launch_cg1(kargs(c, b, sets_cond), L, R, b.f[F_R0 + par], b.f[F_Z0 + par],
+                       b.f[F_Z2 + par], b.f[F_R1 - par], b.f[F_Z1 - par], b.f[F_Z3 - par],
+                       b.f[F_P0], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
+        });
+        return;
+    }
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan(c, R);
+        K(c, TEA_K_UPDATE, sbytes(b, 9), [&] {
+            launch_cg1_update(kargs(c, b), L, R, b.f[F_Z0], b.f[F_Z2], b.f[F_P0], b.f[F_U],
+                              b.f[F_R0], c->stream);
+        });
+    }
+    exchange(c, X_R1, {F_R0});
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan(c, R);
+        K(c, TEA_K_CG1W, sbytes(b, 4), [&] {
+            launch_cg1_w(kargs(c, b, sets_cond), L, R, b.f[F_R0], b.f[F_Z0], b.f[F_KX],
+                         b.f[F_KY], c->stream);
+        });
+    }
+    reduce(c, 0, 3);
+}
+
 void read_state(tea_ctx *c) {
     CK(cudaMemcpyAsync(c->hS, c->blocks[0].S, offsetof(Scalars, cheb_a),
                        cudaMemcpyDeviceToHost, c->stream));
@@ -718,7 +753,7 @@ tea_status map_status(int ds, bool maxed) {
 tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, int s,
                       tea_stats *st) {
     if (c->failed) fail(TEA_ERR_STATE, "context already failed: %s", c->err.c_str());
-    if (method != TEA_CG && method != TEA_CPPCG && method != TEA_BJCG)
+    if (method != TEA_CG && method != TEA_CPPCG && method != TEA_BJCG && method != TEA_CG1)
         fail(TEA_ERR_ARG, "bad method %d", (int)method);
     if (max_iters < 0) fail(TEA_ERR_ARG, "max_iters < 0");
     if (method == TEA_CPPCG && (s < 1 || s > kMaxS))
@@ -756,6 +791,18 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
             });
         reduce(c, 1, 2);
     }
+    if (method == TEA_CG1) {  // w = A r, gam = r.r, del = w.r
+        exchange(c, X_R1, {F_R0});
+        for (auto &b : c->blocks) {
+            Region R = b.owned();
+            Launch L = plan(c, R);
+            K(c, TEA_K_CG1W, sbytes(b, 4), [&] {
+                launch_cg1_w(kargs(c, b), L, R, b.f[F_R0], b.f[F_Z0], b.f[F_KX], b.f[F_KY],
+                             c->stream);
+            });
+        }
+        reduce(c, 0, 3);
+    }
     for (auto &b : c->blocks)
         K(c, TEA_K_SCALAR, 0.0, [&] {
             launch_scalars(kargs(c, b), SC_R0, 0, 0, 0, 0, 0, c->stream);
@@ -770,6 +817,8 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
     if (!c->hS->done) {
         if (method == TEA_BJCG)
             run_loop(c, 3, lim1, [&](int par, bool sc) { body_bj(c, par, sc); });
+        else if (method == TEA_CG1)
+            run_loop(c, 4, lim1, [&](int par, bool sc) { body_cg1(c, par, sc); });
         else
             run_loop(c, 1, lim1, [&](int par, bool sc) { body_cg(c, par, sc); });
     }
@@ -801,7 +850,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         st->presteps = phase2 ? h.presteps : 0;
         st->outer = phase2 ? h.outer : 0;
         st->inner_matvecs = phase2 ? s * (h.outer + 1) : 0;
-        st->matvecs = 1 + h.it + st->inner_matvecs;
+        st->matvecs = 1 + h.it + st->inner_matvecs + (method == TEA_CG1 ? 1 : 0);
         st->status = rs;
         st->r0 = h.r0;
         st->rnorm = std::sqrt(h.red_rr);

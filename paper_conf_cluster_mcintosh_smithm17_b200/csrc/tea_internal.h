@@ -125,6 +125,17 @@ void launch_bj(const KArgs &a, const Region &R, bool update, bool sets_cond, con
                double *r, double *z, const double *ky, const double *bjc, const double *bjd,
                cudaStream_t st);
 
+// Single-reduction (Chronopoulos-Gear) CG. Fused single-block iteration: reads r, w, s
+// (ping-pong) and p, u; writes r', w', s', p, u; one reduction (r.r, w.r).
+void launch_cg1(const KArgs &a, const Launch &L, const Region &R, const double *rin,
+                const double *win, const double *sin, double *rout, double *wout, double *sout,
+                double *p, double *u, const double *kx, const double *ky, cudaStream_t st);
+// Multi-block: pointwise update (s, p, u, r) then w = A r with the dots.
+void launch_cg1_update(const KArgs &a, const Launch &L, const Region &R, const double *w,
+                       double *s, double *p, double *u, double *r, cudaStream_t st);
+void launch_cg1_w(const KArgs &a, const Launch &L, const Region &R, const double *r, double *w,
+                  const double *kx, const double *ky, cudaStream_t st);
+
 // Temporally blocked Chebyshev passes (tea_cheb_tb.cu).
 constexpr int kTbMaxSteps = 5;
 int tb_out_cols(int M);

@@ -345,3 +345,48 @@ def test_bjcg_multiblock(tea, ora, px, py):
     u_g, st_g = gpu_run(tea, deck, dist=dict(px=px, py=py, halo_depth=1, nranks=1), **kw)
     assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
     assert rel_err(u_g, u_o) <= 1e-10
+
+
+# ---------------------------------------------------------------- single-reduction CG (NEXT-2)
+@pytest.mark.parametrize("kind,nx,ny", [("pipe", 128, 128), ("pipe", 256, 200),
+                                        ("random", 300, 203), ("random", 1, 97),
+                                        ("random", 95, 1), ("random", 3, 5)])
+def test_cg1_converged(tea, ora, kind, nx, ny):
+    deck = deck_of(kind, nx, ny, seed=6)
+    kw = dict(method=3, eps=1e-13, max_iters=20000)
+    u_o, st_o, s_o = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, **kw)
+    assert s_o[0] == 0 and st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert field_err(u_g, u_o, kind) <= 1e-10
+
+
+@pytest.mark.parametrize("k", [1, 2, 9])
+def test_cg1_fixed_iterations(tea, ora, k):
+    deck = deck_of("random", 300, 203, seed=8, dt=0.04)
+    kw = dict(method=3, eps=0.0, max_iters=k)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, **kw)
+    assert st_g[0]["iterations"] == k
+    assert field_err(u_g, u_o, "random") <= 1e-12
+
+
+@pytest.mark.parametrize("px,py", [(2, 1), (1, 3), (2, 2), (4, 2)])
+def test_cg1_multiblock(tea, ora, px, py):
+    deck = deck_of("pipe", 200, 170)
+    kw = dict(method=3, eps=1e-13, max_iters=20000)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, dist=dict(px=px, py=py, halo_depth=1, nranks=1), **kw)
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+
+
+@pytest.mark.parametrize("method", [2, 3])
+@pytest.mark.parametrize("loop_mode", [1, 2])
+def test_new_methods_loop_modes_identical(tea, method, loop_mode):
+    deck = deck_of("pipe", 200, 136)
+    ref, st_ref = gpu_run(tea, deck, method=method, eps=1e-12, max_iters=5000)
+    u, st = gpu_run(tea, deck, method=method, eps=1e-12, max_iters=5000, loop_mode=loop_mode,
+                    check_interval=6)
+    assert st[0]["iterations"] == st_ref[0]["iterations"]
+    assert np.array_equal(u, ref)

@@ -171,3 +171,41 @@ def test_not_converged_and_bad_args(ora):
     res = ora.solve(Kx, Ky, u0, method=1, eps=1e-15, max_iters=32, presteps=30)
     assert res.status == 1 and res.stats["outer"] == 2
     assert ora.solve(Kx, Ky, u0, method=1, inner_steps=0).status == -1
+
+
+# ---------------------------------------------------------------- single-reduction CG
+@pytest.mark.parametrize("kind,nx,ny,seed,dt", SMALL)
+def test_cg1_dense_direct_solve(ora, kind, nx, ny, seed, dt):
+    """Chronopoulos-Gear CG (NEXT-2) reaches the dense solution."""
+    d = (inputs.random_fields(nx, ny, seed, dt=dt) if kind == "random"
+         else inputs.crooked_pipe(nx, ny))
+    Kx, Ky, u0 = setup(ora, d)
+    ustar = np.linalg.solve(dense_A(ora, Kx, Ky, nx, ny), u0.ravel()).reshape(ny, nx)
+    res = ora.solve(Kx, Ky, u0, method=ora.CG1, eps=1e-15, max_iters=5000)
+    assert res.status == 0
+    assert np.abs(res.u - ustar).max() / np.abs(ustar).max() <= 1e-11
+
+
+@pytest.mark.parametrize("n", [64, 128])
+def test_cg1_equivalent_to_cg(ora, n):
+    """Same Krylov iterates in exact arithmetic: iteration counts within +-2, fields equal,
+    and the same residual norm after every fixed iteration count (to rounding)."""
+    d = inputs.crooked_pipe(n)
+    Kx, Ky, u0 = setup(ora, d)
+    cg = ora.solve(Kx, Ky, u0, method=ora.CG, eps=1e-13)
+    c1 = ora.solve(Kx, Ky, u0, method=ora.CG1, eps=1e-13)
+    assert abs(cg.stats["iterations"] - c1.stats["iterations"]) <= 2
+    assert np.abs(cg.u - c1.u).max() / np.abs(cg.u).max() <= 1e-11
+    for k in (1, 5, 20):
+        a = ora.solve(Kx, Ky, u0, method=ora.CG, eps=0.0, max_iters=k)
+        b = ora.solve(Kx, Ky, u0, method=ora.CG1, eps=0.0, max_iters=k)
+        assert b.stats["rnorm"] == pytest.approx(a.stats["rnorm"], rel=1e-9)
+        assert np.abs(a.u - b.u).max() / np.abs(a.u).max() <= 1e-12
+
+
+def test_cg1_conservation(ora):
+    d = inputs.crooked_pipe(32)
+    Kx, Ky, u0 = setup(ora, d)
+    for k in (1, 4, 9, 17):
+        res = ora.solve(Kx, Ky, u0, method=ora.CG1, eps=0.0, max_iters=k)
+        assert abs(res.u.sum() - u0.sum()) / u0.sum() <= 1e-13
