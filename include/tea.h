@@ -51,7 +51,15 @@ typedef enum {
  * reduction per iteration, s = A p carried by recurrence -- the restructuring the
  * paper names as future work. Same iterates as CG in
  * exact arithmetic; one fused kernel per iteration on a single block.             */
-typedef enum { TEA_CG = 0, TEA_CPPCG = 1, TEA_BJCG = 2, TEA_CG1 = 3 } tea_method;
+/* TEA_JACOBI / TEA_CHEBY: the stand-alone solvers TeaLeaf ships beside CG
+ * (SURVEY NEXT-4): point Jacobi u += D^{-1} (u^n - A u), and the Chebyshev
+ * iteration (Saad Alg. 12.1) on the interval estimated from `presteps` CG iterations
+ * (as CPPCG). One stencil pass per iteration; the stop test uses the true residual of
+ * the iterate before the last update (reading R19). Chebyshev "cannot cope with some
+ * condition numbers": max_iters bounds it.                          */
+typedef enum {
+    TEA_CG = 0, TEA_CPPCG = 1, TEA_BJCG = 2, TEA_CG1 = 3, TEA_JACOBI = 4, TEA_CHEBY = 5
+} tea_method;
 
 typedef struct tea_ctx tea_ctx; /* opaque, library-owned */
 
@@ -116,6 +124,7 @@ enum {
     TEA_K_TB_FIRST, TEA_K_TB_MID, TEA_K_TB_LAST, /* fused multi-step Chebyshev passes */
     TEA_K_BJ,                                     /* block-Jacobi update + strip solves  */
     TEA_K_CG1, TEA_K_CG1W,                        /* single-reduction CG: fused / A r    */
+    TEA_K_STAT,                                   /* Jacobi / Chebyshev iteration        */
     TEA_K_COUNT
 };
 

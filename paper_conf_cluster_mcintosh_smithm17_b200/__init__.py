@@ -20,12 +20,12 @@ import numpy as np
 
 from . import _build
 
-CG, CPPCG, BJCG, CG1 = 0, 1, 2, 3
+CG, CPPCG, BJCG, CG1, JACOBI, CHEBY = 0, 1, 2, 3, 4, 5
 OK, NOT_CONVERGED = 0, 1
 ERR_ARG, ERR_CUDA, ERR_NCCL, ERR_BREAKDOWN, ERR_STATE = -1, -2, -3, -4, -5
 KERNELS = ["init", "residual", "spmv", "update", "cheb_first", "cheb_step", "cheb_last", "eig",
            "pack", "unpack", "scalar", "tb_first", "tb_mid", "tb_last", "bj", "cg1",
-           "cg1_w"]
+           "cg1_w", "stat"]
 SYMBOLS = ["tea_version", "tea_abi_version", "tea_get_nccl_id", "tea_workspace_bytes", "tea_init",
            "tea_solve", "tea_fetch", "tea_set_u", "tea_kernel_times", "tea_launch_count",
            "tea_finalize", "tea_last_error", "tea_block_extent", "tea_cheb_schedule"]

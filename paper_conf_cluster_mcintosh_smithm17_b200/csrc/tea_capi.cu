@@ -651,6 +651,22 @@ void body_cg1(tea_ctx *c, int par, bool sets_cond) {
     reduce(c, 0, 3);
 }
 
+// Stand-alone Jacobi / Chebyshev iteration: u ping-pongs between U and Z0 (par),
+// the new iterate overwrites u_{k-1} in place; halo of the new iterate exchanged.
+void body_stat(tea_ctx *c, bool cheb, int par, bool sets_cond) {
+    const int in = par ? F_Z0 : F_U, out = par ? F_U : F_Z0;
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan(c, R);
+        K(c, TEA_K_STAT, sbytes(b, cheb ? 6 : 5), [&] {
+            launch_stat(kargs(c, b, sets_cond), L, R, cheb, b.f[in], b.f[F_U0], b.f[out],
+                        b.f[F_KX], b.f[F_KY], c->stream);
+        });
+    }
+    reduce(c, 2, 1);
+    exchange(c, X_U1, {out});
+}
+
 void read_state(tea_ctx *c) {
     CK(cudaMemcpyAsync(c->hS, c->blocks[0].S, offsetof(Scalars, cheb_a),
                        cudaMemcpyDeviceToHost, c->stream));
@@ -753,13 +769,12 @@ tea_status map_status(int ds, bool maxed) {
 tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, int s,
                       tea_stats *st) {
     if (c->failed) fail(TEA_ERR_STATE, "context already failed: %s", c->err.c_str());
-    if (method != TEA_CG && method != TEA_CPPCG && method != TEA_BJCG && method != TEA_CG1)
-        fail(TEA_ERR_ARG, "bad method %d", (int)method);
+    if (method < TEA_CG || method > TEA_CHEBY) fail(TEA_ERR_ARG, "bad method %d", (int)method);
     if (max_iters < 0) fail(TEA_ERR_ARG, "max_iters < 0");
     if (method == TEA_CPPCG && (s < 1 || s > kMaxS))
         fail(TEA_ERR_ARG, "inner_steps must be in [1,%d]", kMaxS);
     const int pre = c->opts.presteps;
-    if (method == TEA_CPPCG && (pre < 1 || pre > kMaxPre))
+    if ((method == TEA_CPPCG || method == TEA_CHEBY) && (pre < 1 || pre > kMaxPre))
         fail(TEA_ERR_ARG, "presteps must be in [1,%d]", kMaxPre);
     c->profiling = c->opts.profile != 0;
 
@@ -767,7 +782,8 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
     CK(cudaStreamWaitEvent(c->stream, c->ev_in, 0));
     CK(cudaEventRecord(c->ev_t0, c->stream));
 
-    const int lim1 = method == TEA_CPPCG ? std::min(pre, max_iters) : max_iters;
+    const bool two_phase = method == TEA_CPPCG || method == TEA_CHEBY;
+    const int lim1 = two_phase ? std::min(pre, max_iters) : max_iters;
     for (auto &b : c->blocks)
         K(c, TEA_K_SCALAR, 0.0, [&] {
             launch_scalars(kargs(c, b), SC_BEGIN, eps, lim1, max_iters, c->opts.eig_margin_lo,
@@ -819,12 +835,34 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
             run_loop(c, 3, lim1, [&](int par, bool sc) { body_bj(c, par, sc); });
         else if (method == TEA_CG1)
             run_loop(c, 4, lim1, [&](int par, bool sc) { body_cg1(c, par, sc); });
+        else if (method == TEA_JACOBI)
+            run_loop(c, 5, lim1, [&](int par, bool sc) { body_stat(c, false, par, sc); });
         else
             run_loop(c, 1, lim1, [&](int par, bool sc) { body_cg(c, par, sc); });
     }
     int ds = c->hS->status;
-    bool phase2 = method == TEA_CPPCG && ds == DS_LIMIT && c->hS->it < max_iters;
-    if (phase2) {
+    if (method == TEA_JACOBI) {  // the final iterate is in Z0 after an odd count
+        if (c->hS->it % 2 == 1)
+            for (auto &b : c->blocks)
+                CK(cudaMemcpyAsync(b.f[F_U] - (size_t)b.L.H * b.L.pitch - b.L.X0,
+                                   b.f[F_Z0] - (size_t)b.L.H * b.L.pitch - b.L.X0,
+                                   b.L.field_bytes, cudaMemcpyDeviceToDevice, c->stream));
+    }
+    bool phase2 = two_phase && ds == DS_LIMIT && c->hS->it < max_iters;
+    if (phase2 && method == TEA_CHEBY) {
+        for (auto &b : c->blocks)
+            K(c, TEA_K_EIG, 0.0, [&] { launch_eig_setup(kargs(c, b), 1, c->stream); });
+        read_state(c);
+        const int pre0 = c->hS->it;
+        if (!c->hS->done)
+            run_loop(c, 6, max_iters, [&](int par, bool sc) { body_stat(c, true, par, sc); });
+        if ((c->hS->it - pre0) % 2 == 1)
+            for (auto &b : c->blocks)
+                CK(cudaMemcpyAsync(b.f[F_U] - (size_t)b.L.H * b.L.pitch - b.L.X0,
+                                   b.f[F_Z0] - (size_t)b.L.H * b.L.pitch - b.L.X0,
+                                   b.L.field_bytes, cudaMemcpyDeviceToDevice, c->stream));
+        ds = c->hS->status;
+    } else if (phase2) {
         // ---- eigen-estimate, coefficients, restart z = B(A) r, p = z
         for (auto &b : c->blocks)
             K(c, TEA_K_EIG, 0.0, [&] { launch_eig_setup(kargs(c, b), s, c->stream); });
@@ -849,7 +887,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         st->iterations = h.it;
         st->presteps = phase2 ? h.presteps : 0;
         st->outer = phase2 ? h.outer : 0;
-        st->inner_matvecs = phase2 ? s * (h.outer + 1) : 0;
+        st->inner_matvecs = phase2 && method == TEA_CPPCG ? s * (h.outer + 1) : 0;
         st->matvecs = 1 + h.it + st->inner_matvecs + (method == TEA_CG1 ? 1 : 0);
         st->status = rs;
         st->r0 = h.r0;

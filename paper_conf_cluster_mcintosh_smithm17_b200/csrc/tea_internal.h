@@ -32,6 +32,7 @@ struct Scalars {
     double theta, eig_min, eig_max, ritz_min, ritz_max;
     double margin_lo, margin_hi;
     double beta_last;
+    double cheb_sigma, cheb_delta, cheb_rho;  // stand-alone Chebyshev solver state
     int it;             // completed iterations (CG + presteps + outer)
     int it_limit;       // iteration limit of the current phase
     int done;           // phase finished (converged / limit / breakdown)
@@ -124,6 +125,11 @@ void launch_bj_setup(const KArgs &a, const Region &R, const double *kx, const do
 void launch_bj(const KArgs &a, const Region &R, bool update, bool sets_cond, const double *w,
                double *r, double *z, const double *ky, const double *bjc, const double *bjd,
                cudaStream_t st);
+
+// Stand-alone Jacobi / Chebyshev iteration: u_k -> u_{k+1} (into uprev_out), ||r_k||^2.
+void launch_stat(const KArgs &a, const Launch &L, const Region &R, bool cheb, const double *uin,
+                 const double *u0, double *uprev_out, const double *kx, const double *ky,
+                 cudaStream_t st);
 
 // Single-reduction (Chronopoulos-Gear) CG. Fused single-block iteration: reads r, w, s
 // (ping-pong) and p, u; writes r', w', s', p, u; one reduction (r.r, w.r).

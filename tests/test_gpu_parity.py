@@ -390,3 +390,39 @@ def test_new_methods_loop_modes_identical(tea, method, loop_mode):
                     check_interval=6)
     assert st[0]["iterations"] == st_ref[0]["iterations"]
     assert np.array_equal(u, ref)
+
+
+# ---------------------------------------------------------------- Jacobi / Chebyshev (NEXT-4)
+@pytest.mark.parametrize("method", [4, 5])
+@pytest.mark.parametrize("kind,nx,ny", [("pipe", 64, 64), ("random", 130, 97), ("random", 1, 40),
+                                        ("random", 33, 1)])
+def test_stationary_converged(tea, ora, method, kind, nx, ny):
+    deck = deck_of(kind, nx, ny, seed=2, dt=0.004)
+    kw = dict(method=method, eps=1e-12, max_iters=200000)
+    u_o, st_o, s_o = ora.run(deck, steps=1, presteps=10, **kw)
+    u_g, st_g = gpu_run(tea, deck, presteps=10, **kw)
+    assert s_o[0] == 0 and st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert field_err(u_g, u_o, kind) <= 1e-10
+
+
+@pytest.mark.parametrize("method,k", [(4, 1), (4, 2), (4, 7), (5, 11), (5, 12), (5, 20)])
+def test_stationary_fixed_iterations(tea, ora, method, k):
+    deck = deck_of("random", 200, 150, seed=3, dt=0.04)
+    kw = dict(method=method, eps=0.0, max_iters=k)
+    u_o, st_o, _ = ora.run(deck, steps=1, presteps=10, **kw)
+    u_g, st_g = gpu_run(tea, deck, presteps=10, **kw)
+    assert st_g[0]["iterations"] == k
+    assert field_err(u_g, u_o, "random") <= 1e-12
+
+
+@pytest.mark.parametrize("method", [4, 5])
+@pytest.mark.parametrize("px,py", [(2, 1), (2, 3)])
+def test_stationary_multiblock(tea, ora, method, px, py):
+    deck = deck_of("pipe", 96, 72)
+    kw = dict(method=method, eps=1e-12, max_iters=200000)
+    u_o, st_o, _ = ora.run(deck, steps=1, presteps=10, **kw)
+    u_g, st_g = gpu_run(tea, deck, presteps=10, dist=dict(px=px, py=py, halo_depth=1, nranks=1),
+                        **kw)
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
