@@ -143,7 +143,7 @@ def run_reference(args):
     oracle.build()
     deck = inputs.crooked_pipe(args.n)
     method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
-              "cg1": oracle.CG1}[args.method]
+              "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY}[args.method]
     sample_iters = args.ref_iters
     for _ in range(args.warmup):  # untimed warm-up (page-in, caches)
         oracle.run(deck, steps=1, method=method, eps=args.eps, max_iters=1,
@@ -176,7 +176,7 @@ def run_reference(args):
 
 
 METHOD_NAME = {"cppcg": "CPPCG", "cg": "CG", "bjcg": "block-Jacobi PCG",
-               "cg1": "single-reduction CG"}
+               "cg1": "single-reduction CG", "jacobi": "Jacobi", "cheby": "Chebyshev"}
 
 
 def metric_name(args):
@@ -189,7 +189,8 @@ def config(args):
                         f"{'CPPCG s=' + str(args.inner) if args.method == 'cppcg' else METHOD_NAME[args.method]}"
                         f" eps={args.eps:g} 1 timestep/step",
             "mesh": [args.n, args.n], "method": args.method, "inner_steps": args.inner,
-            "eps": args.eps, "halo_depth": args.halo_depth, "dt": 0.004,
+            "eps": args.eps, "max_iters": args.max_iters, "halo_depth": args.halo_depth,
+            "dt": 0.004,
             "l2": "inputs larger than L2 (12 fp64 fields x 134 MB at 4096^2)"
             if args.n >= 2048 else "working set fits in L2 (no flush)"}
 
@@ -199,7 +200,7 @@ def cpu_baseline(args, deck):
     import oracle
     oracle.build()
     method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
-              "cg1": oracle.CG1}[args.method]
+              "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY}[args.method]
     t0 = time.perf_counter()
     _, st, _ = oracle.run(deck, steps=1, method=method, eps=args.eps, max_iters=args.ref_iters,
                           inner_steps=args.inner)
@@ -264,7 +265,7 @@ def run_gpu(args):
 
     deck = inputs.crooked_pipe(args.n)
     method = {"cppcg": tea.CPPCG, "cg": tea.CG, "bjcg": tea.BJCG,
-              "cg1": tea.CG1}[args.method]
+              "cg1": tea.CG1, "jacobi": tea.JACOBI, "cheby": tea.CHEBY}[args.method]
     cells = args.n * args.n
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
                 tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode)
@@ -298,6 +299,9 @@ def run_gpu(args):
         model_bytes = sum(5 * 8 * cells + s["presteps"] * cg_iter_bytes(cells) +
                           outer_bytes(cells, args.inner) - 10 * 8 * cells +  # restart chain
                           s["outer"] * outer_bytes(cells, args.inner) for s in stats)
+    elif method in (tea.JACOBI, tea.CHEBY):
+        per = 5 if method == tea.JACOBI else 6
+        model_bytes = len(stats) * 5 * 8 * cells + iters * per * 8 * cells
     elif method == tea.CG1:
         model_bytes = len(stats) * 9 * 8 * cells + iters * 12 * 8 * cells
     elif method == tea.BJCG:
@@ -387,10 +391,12 @@ def main():
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", default="b200", choices=["b200", "reference"])
     ap.add_argument("--n", type=int, default=4096)
-    ap.add_argument("--method", default="cppcg", choices=["cppcg", "cg", "bjcg", "cg1"])
+    ap.add_argument("--method", default="cppcg", choices=["cppcg", "cg", "bjcg", "cg1", "jacobi", "cheby"])
     ap.add_argument("--inner", type=int, default=10)
     ap.add_argument("--eps", type=float, default=1e-12)
-    ap.add_argument("--max-iters", type=int, default=100000)
+    ap.add_argument("--max-iters", type=int, default=0,
+                    help="0 = 100000 (Krylov methods) or 2000 (jacobi/cheby: a fixed-work "
+                         "throughput run; they need O(kappa) iterations at 4096^2)")
     ap.add_argument("--halo-depth", type=int, default=2)
     ap.add_argument("--tile-rows", type=int, default=0)
     ap.add_argument("--tb-steps", type=int, default=0,
@@ -402,6 +408,8 @@ def main():
     args = ap.parse_args()
     if args.warmup < 3:
         ap.error("--warmup must be >= 3")
+    if args.max_iters == 0:
+        args.max_iters = 2000 if args.method in ("jacobi", "cheby") else 100000
     if args.impl == "reference":
         return run_reference(args)
     return run_gpu(args)
