@@ -76,6 +76,10 @@ def lib():
         L.ora_solve_ex.argtypes = [i, i, dp, dp, dp, dp, i, d, i, i, i, i, ip,
                                    C.POINTER(OraStats)]
         L.ora_bj_apply.argtypes = [i, i, dp, dp, i, ip, dp, dp]
+        L.ora_face_coefficients3.argtypes = [i, i, i, d, d, d, dp, i, dp, dp, dp]
+        L.ora_apply_A3.argtypes = [i, i, i, dp, dp, dp, dp, dp]
+        L.ora_solve3.argtypes = [i, i, i, dp, dp, dp, dp, dp, i, d, i, i, i,
+                                 C.POINTER(OraStats)]
         L.ora_timestep.argtypes = [i, i, d, d, d, d, dp, dp, d, i, d, i, i, i, i, dp,
                                    C.POINTER(OraStats)]
         _lib = L
@@ -209,6 +213,55 @@ def run(deck, steps=1, method=CG, eps=1e-10, max_iters=10000, inner_steps=10,
     stats, statuses = [], []
     for _ in range(steps):
         res = solve(Kx, Ky, u, None, method, eps, max_iters, inner_steps, presteps, ybounds)
+        u = res.u
+        stats.append(res.stats)
+        statuses.append(res.status)
+    return u, stats, statuses
+
+
+# --------------------------------------------------------------------------- 3D
+def mesh_r3(deck):
+    """rx, ry, rz = dt/dx^2, dt/dy^2, dt/dz^2."""
+    dx = (deck.xmax - deck.xmin) / deck.nx
+    dy = (deck.ymax - deck.ymin) / deck.ny
+    dz = (deck.zmax - deck.zmin) / deck.nz
+    return deck.dt / (dx * dx), deck.dt / (dy * dy), deck.dt / (dz * dz)
+
+
+def face_coefficients3(nx, ny, nz, rx, ry, rz, rho, mean_mode=0):
+    Kx = np.zeros((nz, ny, nx + 1))
+    Ky = np.zeros((nz, ny + 1, nx))
+    Kz = np.zeros((nz + 1, ny, nx))
+    lib().ora_face_coefficients3(nx, ny, nz, rx, ry, rz, _c(rho), mean_mode, Kx, Ky, Kz)
+    return Kx, Ky, Kz
+
+
+def apply_A3(Kx, Ky, Kz, p):
+    nz, ny, nx = p.shape
+    w = np.zeros((nz, ny, nx))
+    lib().ora_apply_A3(nx, ny, nz, _c(Kx), _c(Ky), _c(Kz), _c(p), w)
+    return w
+
+
+def solve3(Kx, Ky, Kz, u0, u_init=None, method=CG, eps=1e-10, max_iters=10000, inner_steps=10,
+           presteps=PRESTEPS):
+    nz, ny, nx = u0.shape
+    u = _c(u0 if u_init is None else u_init).copy()
+    st = OraStats()
+    s = lib().ora_solve3(nx, ny, nz, _c(Kx), _c(Ky), _c(Kz), _c(u0), u, method, eps, max_iters,
+                         inner_steps, presteps, C.byref(st))
+    return Result(u, s, st.as_dict())
+
+
+def run3(deck, steps=1, method=CG, eps=1e-10, max_iters=10000, inner_steps=10,
+         presteps=PRESTEPS, mean_mode=0):
+    rx, ry, rz = mesh_r3(deck)
+    Kx, Ky, Kz = face_coefficients3(deck.nx, deck.ny, deck.nz, rx, ry, rz, deck.density,
+                                    mean_mode)
+    u = _c(deck.density) * _c(deck.energy)
+    stats, statuses = [], []
+    for _ in range(steps):
+        res = solve3(Kx, Ky, Kz, u, None, method, eps, max_iters, inner_steps, presteps)
         u = res.u
         stats.append(res.stats)
         statuses.append(res.status)

@@ -33,7 +33,8 @@ from dataclasses import dataclass, field
 
 import numpy as np
 
-__all__ = ["Deck", "crooked_pipe", "random_fields", "uniform_fields", "deck"]
+__all__ = ["Deck", "Deck3", "crooked_pipe", "random_fields", "uniform_fields", "deck",
+           "crooked_pipe3", "random_fields3", "uniform_fields3"]
 
 
 @dataclass
@@ -121,3 +122,64 @@ def deck(kind: str, nx: int, ny: int | None = None, seed: int = 0, **kw) -> Deck
     if kind == "uniform":
         return uniform_fields(nx, ny, seed=seed, **kw)
     raise ValueError(f"unknown deck kind {kind!r}")
+
+
+# ------------------------------------------------------------------ 3D
+@dataclass
+class Deck3:
+    """A 3D problem: fields of shape (nz, ny, nx), index (l*ny + k)*nx + j."""
+
+    nx: int
+    ny: int
+    nz: int
+    xmin: float
+    xmax: float
+    ymin: float
+    ymax: float
+    zmin: float
+    zmax: float
+    dt: float
+    density: np.ndarray = field(repr=False)
+    energy: np.ndarray = field(repr=False)
+    name: str = ""
+
+
+def crooked_pipe3(nx: int, ny: int | None = None, nz: int | None = None) -> Deck3:
+    """The 2D crooked-pipe states extruded along z over [0,10], plus a vertical leg
+    [5,6)x[7,8)x[0,10) -> z in [2,10) connecting the outlet upward (reading R20: the
+    paper gives no 3D deck; this keeps the pipe 'crooked' in all three directions)."""
+    ny = nx if ny is None else ny
+    nz = nx if nz is None else nz
+    lo, hi = 0.0, 10.0
+    xc = lo + (np.arange(nx) + 0.5) * (hi - lo) / nx
+    yc = lo + (np.arange(ny) + 0.5) * (hi - lo) / ny
+    zc = lo + (np.arange(nz) + 0.5) * (hi - lo) / nz
+    Z, Y, X = np.meshgrid(zc, yc, xc, indexing="ij")
+    rho = np.full((nz, ny, nx), PIPE_BACKGROUND[0])
+    e = np.full((nz, ny, nx), PIPE_BACKGROUND[1])
+    slab = (Z >= 0.0) & (Z < 2.0)
+    for x0, x1, y0, y1, r, en in PIPE_STATES:
+        m = (X >= x0) & (X < x1) & (Y >= y0) & (Y < y1) & slab
+        rho[m] = r
+        e[m] = en
+    m = (X >= 5.0) & (X < 6.0) & (Y >= 7.0) & (Y < 8.0) & (Z >= 2.0) & (Z < 10.0)
+    rho[m] = 0.1
+    e[m] = 0.1
+    return Deck3(nx, ny, nz, lo, hi, lo, hi, lo, hi, PIPE_DT, np.ascontiguousarray(rho),
+                 np.ascontiguousarray(e), name=f"crooked_pipe3_{nx}x{ny}x{nz}")
+
+
+def random_fields3(nx: int, ny: int, nz: int, seed: int = 0, dt: float = 0.004) -> Deck3:
+    rng = np.random.default_rng(seed)
+    rho = np.exp(rng.uniform(np.log(0.1), np.log(100.0), size=(nz, ny, nx)))
+    e = rng.uniform(1.0e-3, 25.0, size=(nz, ny, nx))
+    return Deck3(nx, ny, nz, 0.0, 10.0, 0.0, 10.0, 0.0, 10.0, dt, np.ascontiguousarray(rho),
+                 np.ascontiguousarray(e), name=f"random3_{nx}x{ny}x{nz}_s{seed}")
+
+
+def uniform_fields3(nx: int, ny: int, nz: int, rho: float = 1.0, seed: int = 0,
+                    dt: float = 0.004, extent=(0.0, 10.0, 0.0, 10.0, 0.0, 10.0)) -> Deck3:
+    rng = np.random.default_rng(seed)
+    e = rng.uniform(1.0e-3, 25.0, size=(nz, ny, nx))
+    return Deck3(nx, ny, nz, *extent, dt, np.full((nz, ny, nx), float(rho)),
+                 np.ascontiguousarray(e), name=f"uniform3_{nx}x{ny}x{nz}")
