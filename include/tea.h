@@ -63,11 +63,16 @@ typedef enum {
 
 typedef struct tea_ctx tea_ctx; /* opaque, library-owned */
 
-/* Mesh: nx x ny cells on [xmin,xmax] x [ymin,ymax]; dx = (xmax-xmin)/nx,
- * dy = (ymax-ymin)/ny; rx = dt/dx^2, ry = dt/dy^2 (BASELINE.json north_star). */
+/* Mesh: nx x ny (x nz) cells on [xmin,xmax] x [ymin,ymax] (x [zmin,zmax]);
+ * dx = (xmax-xmin)/nx, ...; rx = dt/dx^2, ry = dt/dy^2 (BASELINE.json north_star),
+ * rz = dt/dz^2. nz <= 1: the 2D 5-point problem (Listing 1); nz > 1: the 3D 7-point
+ * problem (reading R20) -- single block, methods CG, CPPCG,
+ * CG1, JACOBI, CHEBY. 3D host arrays are nx*ny*nz, index (l*ny + k)*nx + j.        */
 typedef struct {
     int nx, ny;
     double xmin, xmax, ymin, ymax;
+    int nz;
+    double zmin, zmax;
 } tea_mesh;
 
 /* Decomposition: px x py blocks, block b = by*px + bx owns the

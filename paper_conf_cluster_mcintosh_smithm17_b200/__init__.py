@@ -39,7 +39,8 @@ class TeaError(RuntimeError):
 
 class Mesh(C.Structure):
     _fields_ = [("nx", C.c_int), ("ny", C.c_int), ("xmin", C.c_double), ("xmax", C.c_double),
-                ("ymin", C.c_double), ("ymax", C.c_double)]
+                ("ymin", C.c_double), ("ymax", C.c_double), ("nz", C.c_int),
+                ("zmin", C.c_double), ("zmax", C.c_double)]
 
 
 class Dist(C.Structure):
@@ -107,12 +108,16 @@ def version() -> str:
     return lib().tea_version().decode()
 
 
-def make_mesh(nx, ny, xmin=0.0, xmax=10.0, ymin=0.0, ymax=10.0) -> Mesh:
-    return Mesh(nx, ny, xmin, xmax, ymin, ymax)
+def make_mesh(nx, ny, xmin=0.0, xmax=10.0, ymin=0.0, ymax=10.0, nz=1, zmin=0.0,
+              zmax=1.0) -> Mesh:
+    return Mesh(nx, ny, xmin, xmax, ymin, ymax, nz, zmin, zmax)
 
 
 def mesh_of(deck) -> Mesh:
-    return Mesh(deck.nx, deck.ny, deck.xmin, deck.xmax, deck.ymin, deck.ymax)
+    """Mesh of a 2D Deck or a 3D Deck3 (inputs.py)."""
+    nz = getattr(deck, "nz", 1)
+    return Mesh(deck.nx, deck.ny, deck.xmin, deck.xmax, deck.ymin, deck.ymax, nz,
+                getattr(deck, "zmin", 0.0), getattr(deck, "zmax", 1.0))
 
 
 def workspace_bytes(mesh: Mesh, dist: Dist | None = None) -> int:
@@ -196,7 +201,7 @@ class Tea:
             self.stream = stream if stream is not None else torch.cuda.current_stream(self.device)
             rho, prho = _f64(density)
             en, pen = _f64(energy)
-            assert rho.size == mesh.nx * mesh.ny and en.size == rho.size
+            assert rho.size == mesh.nx * mesh.ny * max(mesh.nz, 1) and en.size == rho.size
             ctx = C.c_void_p()
             st = self.L.tea_init(C.byref(ctx), C.byref(mesh), prho, pen, float(dt),
                                  C.byref(self._dist) if self._dist else None, C.byref(self.opts),
@@ -218,7 +223,8 @@ class Tea:
 
     def fetch(self, out=None):
         if out is None:
-            out = np.zeros((self.mesh.ny, self.mesh.nx))
+            shape = ((self.mesh.nz,) if self.mesh.nz > 1 else ()) + (self.mesh.ny, self.mesh.nx)
+            out = np.zeros(shape)
         assert out.flags.c_contiguous and out.dtype == np.float64
         st = self.L.tea_fetch(self.ctx, out.ctypes.data_as(C.c_void_p))
         if st != OK:

@@ -44,7 +44,9 @@ struct XPlan {
 
 struct BlockLayout {
     int bi, bj, gx0, gx1, gy0, gy1, bx, by;
-    int H, X0, pitch, rows;
+    int nz;          // planes (1: 2D)
+    long long ps;    // plane stride (doubles), rows * pitch
+    int H, X0, pitch, rows, planes;
     size_t field_bytes, scalars_off, partials_off, partials_cap, boxes_off, halo_off,
         halo_cap, total;
     bool has_nbr;
@@ -68,11 +70,15 @@ BlockLayout layout_block(const tea_mesh &m, int px, int py, int d, int b) {
     L.X0 = (int)round_up(d + 4, 16);
     L.pitch = (int)round_up(L.X0 + L.bx + d + 4, 32);
     L.rows = L.by + 2 * L.H;
-    L.field_bytes = round_up((size_t)L.rows * L.pitch * sizeof(double), 256);
+    L.nz = m.nz > 1 ? m.nz : 1;
+    L.ps = (long long)L.rows * L.pitch;
+    L.planes = L.nz > 1 ? L.nz + 2 * L.H : 1;
+    L.field_bytes = round_up((size_t)L.planes * L.ps * sizeof(double), 256);
     size_t off = L.field_bytes * F_COUNT;
     L.scalars_off = off;
     off += round_up(sizeof(Scalars), 256);
-    L.partials_cap = 2 * (size_t)max_ctas(L.bx + 2 * d + 2, L.by + 2 * d + 2);
+    L.partials_cap = 2 * (size_t)std::max(max_ctas(L.bx + 2 * d + 2, L.by + 2 * d + 2),
+                                          L.nz > 1 ? max_ctas3(L.bx, L.by, L.nz) : 0);
     L.partials_off = off;
     off += round_up(L.partials_cap * sizeof(double), 256);
     L.has_nbr = (px * py > 1);
@@ -179,6 +185,9 @@ KArgs kargs(tea_ctx *c, const BlockCtx &b, bool set_cond = false) {
     a.partials = b.partials;
     a.cond = c->cond;
     a.set_cond = set_cond ? 1 : 0;
+    a.kz = b.f[F_KZ];
+    a.ps = b.L.ps;
+    a.nz = b.L.nz;
     return a;
 }
 
@@ -223,6 +232,17 @@ void resolve_profile(tea_ctx *c) {
 
 Launch plan(tea_ctx *c, const Region &R) {
     return plan_stencil(R, c->opts.tile_rows > 0 ? c->opts.tile_rows : c->ty_override, 1184);
+}
+// stencil kernels: 2D march over rows, or the 3D march over planes
+Launch plan_st(tea_ctx *c, const BlockCtx &b, const Region &R) {
+    if (b.L.nz > 1) return plan_stencil3(R, b.L.nz, c->opts.tile_rows);
+    return plan(c, R);
+}
+// pointwise kernels: the 2D tiling of one plane, planes on grid.z
+Launch plan_pw(tea_ctx *c, const BlockCtx &b, const Region &R) {
+    Launch L = plan(c, R);
+    L.grid.z = b.L.nz;
+    return L;
 }
 
 // ------------------------------------------------------------------ reductions
@@ -422,15 +442,20 @@ std::vector<ChebOpS> cheb_schedule(int s, int d) {
 // ------------------------------------------------------------------ phase bodies
 int zbuf(int i) { return F_Z0 + ((i - 1) % 3); }  // per-step path: z_i lives in Z[(i-1)%3]
 
+// start of a field's allocation (orig points at cell (0,0,0))
+double *field_base(const BlockCtx &b, int f) {
+    return b.f[f] - (b.L.nz > 1 ? (size_t)b.L.H * b.L.ps : 0) - (size_t)b.L.H * b.L.pitch - b.L.X0;
+}
+
 // algorithmic bytes of a launch: streams x 8 B x owned cells
 double sbytes(const BlockCtx &b, int streams) {
-    return 8.0 * streams * (double)b.L.bx * (double)b.L.by;
+    return 8.0 * streams * (double)b.L.bx * (double)b.L.by * (double)b.L.nz;
 }
 
 void body_cg(tea_ctx *c, int par, bool last_sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
-        Launch L = plan(c, R);
+        Launch L = plan_st(c, b, R);
         K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[F_R0], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
@@ -439,7 +464,7 @@ void body_cg(tea_ctx *c, int par, bool last_sets_cond) {
     reduce(c, 0, 1);
     for (auto &b : c->blocks) {
         Region R = b.owned();
-        Launch L = plan(c, R);
+        Launch L = plan_pw(c, b, R);
         K(c, TEA_K_UPDATE, sbytes(b, 3), [&] {
             launch_update(kargs(c, b, last_sets_cond), L, R, b.f[F_W], b.f[F_R0], c->stream);
         });
@@ -470,7 +495,7 @@ int cheb_chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, b
             for (auto &b : c->blocks) {
                 Region R = b.ext(op.arg);
                 Region D = b.owned();
-                Launch L = plan(c, R);
+                Launch L = plan_st(c, b, R);
                 const bool fu = fused && step == 1;
                 const double *z1 = step >= 2 ? b.f[zbuf(step - 1)] : nullptr;
                 const double *z2 = step >= 3 ? b.f[zbuf(step - 2)] : nullptr;
@@ -552,16 +577,17 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
 }
 
 bool single_block(tea_ctx *c) { return c->px * c->py == 1; }
+bool is3d(const tea_ctx *c) { return c->blocks[0].L.nz > 1; }
 
 int chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond) {
-    if (single_block(c) && tb_steps(c) > 1)
+    if (single_block(c) && !is3d(c) && tb_steps(c) > 1)
         return cheb_chain_tb(c, s, restart, fused, rin, rout, sets_cond);
     return cheb_chain(c, s, restart, fused, rin, rout, sets_cond);
 }
 
 // field holding z_s after a chain (same for every chain of a context and s)
 int zs_field(tea_ctx *c, int s) {
-    if (single_block(c) && tb_steps(c) > 1) {
+    if (single_block(c) && !is3d(c) && tb_steps(c) > 1) {
         const int P = (int)tb_passes(s, tb_steps(c)).size();
         return (P - 1) % 2 == 0 ? F_Z1 : F_Z3;
     }
@@ -573,7 +599,7 @@ void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
     const int zs = zs_field(c, s);
     for (auto &b : c->blocks) {
         Region R = b.owned();
-        Launch L = plan(c, R);
+        Launch L = plan_st(c, b, R);
         K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[zs], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
@@ -585,7 +611,7 @@ void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
     } else {
         for (auto &b : c->blocks) {
             Region R = b.owned();
-            Launch L = plan(c, R);
+            Launch L = plan_pw(c, b, R);
             K(c, TEA_K_UPDATE, sbytes(b, 3), [&] {
                 launch_update_nodot(kargs(c, b), L, R, b.f[F_W], b.f[F_R0], c->stream);
             });
@@ -598,7 +624,7 @@ void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
 void body_bj(tea_ctx *c, int par, bool sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
-        Launch L = plan(c, R);
+        Launch L = plan_st(c, b, R);
         K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[F_Z0], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
@@ -623,7 +649,7 @@ void body_cg1(tea_ctx *c, int par, bool sets_cond) {
     if (single_block(c)) {
         BlockCtx &b = c->blocks[0];
         Region R = b.owned();
-        Launch L = plan(c, R);
+        Launch L = plan_st(c, b, R);
         K(c, TEA_K_CG1, sbytes(b, 12), [&] {
             launch_cg1(kargs(c, b, sets_cond), L, R, b.f[F_R0 + par], b.f[F_Z0 + par],
                        b.f[F_Z2 + par], b.f[F_R1 - par], b.f[F_Z1 - par], b.f[F_Z3 - par],
@@ -633,7 +659,7 @@ void body_cg1(tea_ctx *c, int par, bool sets_cond) {
     }
     for (auto &b : c->blocks) {
         Region R = b.owned();
-        Launch L = plan(c, R);
+        Launch L = plan_pw(c, b, R);
         K(c, TEA_K_UPDATE, sbytes(b, 9), [&] {
             launch_cg1_update(kargs(c, b), L, R, b.f[F_Z0], b.f[F_Z2], b.f[F_P0], b.f[F_U],
                               b.f[F_R0], c->stream);
@@ -642,7 +668,7 @@ void body_cg1(tea_ctx *c, int par, bool sets_cond) {
     exchange(c, X_R1, {F_R0});
     for (auto &b : c->blocks) {
         Region R = b.owned();
-        Launch L = plan(c, R);
+        Launch L = plan_st(c, b, R);
         K(c, TEA_K_CG1W, sbytes(b, 4), [&] {
             launch_cg1_w(kargs(c, b, sets_cond), L, R, b.f[F_R0], b.f[F_Z0], b.f[F_KX],
                          b.f[F_KY], c->stream);
@@ -657,7 +683,7 @@ void body_stat(tea_ctx *c, bool cheb, int par, bool sets_cond) {
     const int in = par ? F_Z0 : F_U, out = par ? F_U : F_Z0;
     for (auto &b : c->blocks) {
         Region R = b.owned();
-        Launch L = plan(c, R);
+        Launch L = plan_st(c, b, R);
         K(c, TEA_K_STAT, sbytes(b, cheb ? 6 : 5), [&] {
             launch_stat(kargs(c, b, sets_cond), L, R, cheb, b.f[in], b.f[F_U0], b.f[out],
                         b.f[F_KX], b.f[F_KY], c->stream);
@@ -770,6 +796,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
                       tea_stats *st) {
     if (c->failed) fail(TEA_ERR_STATE, "context already failed: %s", c->err.c_str());
     if (method < TEA_CG || method > TEA_CHEBY) fail(TEA_ERR_ARG, "bad method %d", (int)method);
+    if (method == TEA_BJCG && is3d(c)) fail(TEA_ERR_ARG, "block Jacobi is 2D only");
     if (max_iters < 0) fail(TEA_ERR_ARG, "max_iters < 0");
     if (method == TEA_CPPCG && (s < 1 || s > kMaxS))
         fail(TEA_ERR_ARG, "inner_steps must be in [1,%d]", kMaxS);
@@ -792,7 +819,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
     exchange(c, X_U1, {F_U});
     for (auto &b : c->blocks) {
         Region R = b.owned();
-        Launch L = plan(c, R);
+        Launch L = plan_st(c, b, R);
         K(c, TEA_K_RESIDUAL, sbytes(b, 5), [&] {
             launch_residual(kargs(c, b), L, R, b.f[F_U], b.f[F_KX], b.f[F_KY], b.f[F_U0],
                             b.f[F_R0], c->stream);
@@ -811,7 +838,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         exchange(c, X_R1, {F_R0});
         for (auto &b : c->blocks) {
             Region R = b.owned();
-            Launch L = plan(c, R);
+            Launch L = plan_st(c, b, R);
             K(c, TEA_K_CG1W, sbytes(b, 4), [&] {
                 launch_cg1_w(kargs(c, b), L, R, b.f[F_R0], b.f[F_Z0], b.f[F_KX], b.f[F_KY],
                              c->stream);
@@ -844,9 +871,8 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
     if (method == TEA_JACOBI) {  // the final iterate is in Z0 after an odd count
         if (c->hS->it % 2 == 1)
             for (auto &b : c->blocks)
-                CK(cudaMemcpyAsync(b.f[F_U] - (size_t)b.L.H * b.L.pitch - b.L.X0,
-                                   b.f[F_Z0] - (size_t)b.L.H * b.L.pitch - b.L.X0,
-                                   b.L.field_bytes, cudaMemcpyDeviceToDevice, c->stream));
+                CK(cudaMemcpyAsync(field_base(b, F_U), field_base(b, F_Z0), b.L.field_bytes,
+                                   cudaMemcpyDeviceToDevice, c->stream));
     }
     bool phase2 = two_phase && ds == DS_LIMIT && c->hS->it < max_iters;
     if (phase2 && method == TEA_CHEBY) {
@@ -858,9 +884,8 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
             run_loop(c, 6, max_iters, [&](int par, bool sc) { body_stat(c, true, par, sc); });
         if ((c->hS->it - pre0) % 2 == 1)
             for (auto &b : c->blocks)
-                CK(cudaMemcpyAsync(b.f[F_U] - (size_t)b.L.H * b.L.pitch - b.L.X0,
-                                   b.f[F_Z0] - (size_t)b.L.H * b.L.pitch - b.L.X0,
-                                   b.L.field_bytes, cudaMemcpyDeviceToDevice, c->stream));
+                CK(cudaMemcpyAsync(field_base(b, F_U), field_base(b, F_Z0), b.L.field_bytes,
+                                   cudaMemcpyDeviceToDevice, c->stream));
         ds = c->hS->status;
     } else if (phase2) {
         // ---- eigen-estimate, coefficients, restart z = B(A) r, p = z
@@ -942,6 +967,14 @@ static tea_status check_decomp(const tea_mesh *m, const tea_dist *dist, int *px,
         *why = "multi-process runs need exactly one block per rank (px*py == nranks)";
         return TEA_ERR_ARG;
     }
+    if (m->nz > 1 && (*px * *py != 1 || *nranks != 1)) {
+        *why = "3D meshes run on a single block (px = py = nranks = 1)";
+        return TEA_ERR_ARG;
+    }
+    if (m->nz > 1 && !(m->zmax > m->zmin)) {
+        *why = "bad z extent";
+        return TEA_ERR_ARG;
+    }
     if (*px * *py > 64) {
         *why = "at most 64 blocks";
         return TEA_ERR_ARG;
@@ -1017,7 +1050,8 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
         // capture target: multi-process runs use chunked graphs (same kernels).
         if (nranks > 1 && o.loop_mode == 0) o.loop_mode = 1;
         c->opts = o;
-        for (long long i = 0; i < (long long)mesh->nx * mesh->ny; i += 1 + ((long long)mesh->nx * mesh->ny) / 4096)
+        const long long ncell = (long long)mesh->nx * mesh->ny * (mesh->nz > 1 ? mesh->nz : 1);
+        for (long long i = 0; i < ncell; i += 1 + ncell / 4096)
             if (!(density[i] > 0.0)) fail(TEA_ERR_ARG, "density must be > 0");
 
         c->user_stream = (cudaStream_t)cuda_stream;
@@ -1047,7 +1081,8 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
             b.L = layout_block(*mesh, px, py, d, b.id);
             const BlockLayout &L = b.L;
             for (int f = 0; f < F_COUNT; ++f)
-                b.f[f] = (double *)(ws + f * L.field_bytes) + (size_t)L.H * L.pitch + L.X0;
+                b.f[f] = (double *)(ws + f * L.field_bytes) + (L.nz > 1 ? (size_t)L.H * L.ps : 0) +
+                         (size_t)L.H * L.pitch + L.X0;
             b.S = (Scalars *)(ws + L.scalars_off);
             b.partials = (double *)(ws + L.partials_off);
             for (int dd = 0; dd < kNDir; ++dd) {
@@ -1059,6 +1094,29 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
                 b.sendbuf = (double *)(ws + L.halo_off);
                 b.recvbuf = (double *)(ws + L.halo_off + round_up(L.halo_cap * sizeof(double), 256));
                 build_xplans(c.get(), b, (int *)(ws + L.boxes_off));
+            }
+            if (L.nz > 1) {  // 3D, single block: stage plane by plane, zero margins
+                const size_t hp = (size_t)mesh->nx * sizeof(double);
+                const size_t plane = (size_t)mesh->nx * mesh->ny;
+                for (int l = 0; l < L.nz; ++l) {
+                    CK(cudaMemcpy2DAsync(b.f[F_W] + l * L.ps, L.pitch * sizeof(double),
+                                         density + l * plane, hp, hp, mesh->ny,
+                                         cudaMemcpyHostToDevice, c->stream));
+                    CK(cudaMemcpy2DAsync(b.f[F_Z0] + l * L.ps, L.pitch * sizeof(double),
+                                         energy + l * plane, hp, hp, mesh->ny,
+                                         cudaMemcpyHostToDevice, c->stream));
+                }
+                const double dz = (mesh->zmax - mesh->zmin) / mesh->nz;
+                K(c.get(), TEA_K_INIT, 0.0, [&] {
+                    launch_init_fields3(kargs(c.get(), b), b.f[F_W], b.f[F_Z0], b.f[F_U0],
+                                        b.f[F_U], b.f[F_KX], b.f[F_KY], b.f[F_KZ], L.bx, L.by,
+                                        L.nz, c->rx, c->ry, dt / (dz * dz), o.mean_mode,
+                                        c->stream);
+                });
+                CK(cudaMemsetAsync(ws + F_W * L.field_bytes, 0, L.field_bytes, c->stream));
+                CK(cudaMemsetAsync(ws + F_Z0 * L.field_bytes, 0, L.field_bytes, c->stream));
+                ws += L.total;
+                continue;
             }
             // stage rho -> W, e -> Z0 over the block plus margin m (clipped to the mesh)
             const int m = d + 1;
@@ -1121,9 +1179,12 @@ tea_status tea_fetch(tea_ctx *ctx, double *u_host) {
         if (ctx->failed) fail(TEA_ERR_STATE, "context failed: %s", ctx->err.c_str());
         for (auto &b : ctx->blocks) {
             const BlockLayout &L = b.L;
-            CK(cudaMemcpy2DAsync(u_host + (size_t)L.gy0 * ctx->mesh.nx + L.gx0,
-                                 ctx->mesh.nx * sizeof(double), b.f[F_U], L.pitch * sizeof(double),
-                                 L.bx * sizeof(double), L.by, cudaMemcpyDeviceToHost, ctx->stream));
+            const size_t plane = (size_t)ctx->mesh.nx * ctx->mesh.ny;
+            for (int l = 0; l < L.nz; ++l)
+                CK(cudaMemcpy2DAsync(u_host + l * plane + (size_t)L.gy0 * ctx->mesh.nx + L.gx0,
+                                     ctx->mesh.nx * sizeof(double), b.f[F_U] + l * L.ps,
+                                     L.pitch * sizeof(double), L.bx * sizeof(double), L.by,
+                                     cudaMemcpyDeviceToHost, ctx->stream));
         }
         CK(cudaStreamSynchronize(ctx->stream));
         return TEA_OK;
@@ -1139,10 +1200,12 @@ tea_status tea_set_u(tea_ctx *ctx, const double *u_host) {
         if (ctx->failed) fail(TEA_ERR_STATE, "context failed: %s", ctx->err.c_str());
         for (auto &b : ctx->blocks) {
             const BlockLayout &L = b.L;
-            CK(cudaMemcpy2DAsync(b.f[F_U], L.pitch * sizeof(double),
-                                 u_host + (size_t)L.gy0 * ctx->mesh.nx + L.gx0,
-                                 ctx->mesh.nx * sizeof(double), L.bx * sizeof(double), L.by,
-                                 cudaMemcpyHostToDevice, ctx->stream));
+            const size_t plane = (size_t)ctx->mesh.nx * ctx->mesh.ny;
+            for (int l = 0; l < L.nz; ++l)
+                CK(cudaMemcpy2DAsync(b.f[F_U] + l * L.ps, L.pitch * sizeof(double),
+                                     u_host + l * plane + (size_t)L.gy0 * ctx->mesh.nx + L.gx0,
+                                     ctx->mesh.nx * sizeof(double), L.bx * sizeof(double), L.by,
+                                     cudaMemcpyHostToDevice, ctx->stream));
         }
         CK(cudaStreamSynchronize(ctx->stream));
         return TEA_OK;

@@ -57,7 +57,7 @@ struct Region {
 
 // Field indices inside a block's workspace.
 enum Field {
-    F_U0 = 0, F_U, F_KX, F_KY, F_R0, F_R1, F_P0, F_P1, F_W, F_Z0, F_Z1, F_Z2, F_Z3,
+    F_U0 = 0, F_U, F_KX, F_KY, F_KZ, F_R0, F_R1, F_P0, F_P1, F_W, F_Z0, F_Z1, F_Z2, F_Z3,
     F_BJC, F_BJD,  // block-Jacobi Thomas coefficients c'_i and 1/den_i
     F_COUNT
 };
@@ -78,9 +78,17 @@ struct KArgs {
     double *partials;
     cudaGraphConditionalHandle cond;  // WHILE-loop handle (0 = none)
     int set_cond;                     // this launch may end the WHILE loop
+    // 3D: planes of (rows x pitch), plane stride ps; nz == 1 is 2D
+    const double *kz;
+    long long ps;
+    int nz;
 };
 
 Launch plan_stencil(const Region &R, int ty_req, int ncta_target);
+// 3D stencil geometry: CTA = 4 warps on 4 consecutive rows of one 64-column strip,
+// marching tz planes (grid = strips x rows/4 x planes/tz).
+Launch plan_stencil3(const Region &R, int nz, int tz_req);
+int max_ctas3(int width, int height, int nz);
 Launch plan_pointwise(const Region &R, int ty_req, int ncta_target);
 int max_ctas(int width, int height);
 
@@ -88,6 +96,10 @@ void launch_init_fields(const KArgs &a, const double *rho, const double *en, dou
                         double *u, double *kx, double *ky, Region owned, Region all,
                         Region kxr, Region kyr, double rx, double ry, int mean_mode,
                         cudaStream_t st);
+// 3D: Kx, Ky, Kz (rz = dt/dz^2) and u0 = u = rho e on the single block (planes [0, nz))
+void launch_init_fields3(const KArgs &a, const double *rho, const double *en, double *u0,
+                         double *u, double *kx, double *ky, double *kz, int nx, int ny, int nz,
+                         double rx, double ry, double rz, int mean_mode, cudaStream_t st);
 void launch_residual(const KArgs &a, const Launch &L, const Region &R, const double *u,
                      const double *kx, const double *ky, double *u0, double *r,
                      cudaStream_t st);

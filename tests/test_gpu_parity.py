@@ -426,3 +426,44 @@ def test_stationary_multiblock(tea, ora, method, px, py):
                         **kw)
     assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
     assert rel_err(u_g, u_o) <= 1e-10
+
+
+# ---------------------------------------------------------------- 3D (NEXT-4)
+def deck3_of(kind, nx, ny, nz, seed=0, dt=0.004):
+    from paper_conf_cluster_mcintosh_smithm17_b200 import inputs
+    if kind == "pipe":
+        return inputs.crooked_pipe3(nx, ny, nz)
+    return inputs.random_fields3(nx, ny, nz, seed, dt=dt)
+
+
+@pytest.mark.parametrize("method", [0, 1, 3, 4, 5])
+@pytest.mark.parametrize("kind,nx,ny,nz", [("pipe", 40, 36, 28), ("random", 33, 17, 9),
+                                           ("random", 70, 5, 2)])
+def test_3d_converged(tea, ora, method, kind, nx, ny, nz):
+    deck = deck3_of(kind, nx, ny, nz, seed=1)
+    kw = dict(method=method, eps=1e-12, max_iters=200000, inner_steps=6)
+    u_o, st_o, s_o = ora.run3(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, **kw)
+    assert s_o[0] == 0 and st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert field_err(u_g, u_o, kind) <= 1e-10
+
+
+@pytest.mark.parametrize("method,k", [(0, 3), (1, 33), (3, 4), (4, 5), (5, 35)])
+def test_3d_fixed_iterations(tea, ora, method, k):
+    deck = deck3_of("random", 45, 23, 11, seed=2, dt=0.04)
+    kw = dict(method=method, eps=0.0, max_iters=k, inner_steps=5)
+    u_o, st_o, _ = ora.run3(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, **kw)
+    assert st_g[0]["iterations"] == k
+    assert field_err(u_g, u_o, "random") <= 1e-12
+
+
+def test_3d_rejections(tea):
+    deck = deck3_of("random", 16, 16, 8)
+    with pytest.raises(tea.TeaError):
+        tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt,
+                dist=dict(px=2, py=1, nranks=1))
+    t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt)
+    assert t.solve(method=2, raise_on_error=False).status == tea.ERR_ARG  # block Jacobi: 2D
+    t.close()
