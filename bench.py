@@ -141,18 +141,18 @@ def run_reference(args):
     if rank != 0:
         return 0
     oracle.build()
-    deck = inputs.crooked_pipe(args.n)
+    deck = make_deck(args)
     method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
               "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY}[args.method]
     sample_iters = args.ref_iters
+    orun = oracle.run3 if args.nz > 1 else oracle.run
     for _ in range(args.warmup):  # untimed warm-up (page-in, caches)
-        oracle.run(deck, steps=1, method=method, eps=args.eps, max_iters=1,
-                   inner_steps=args.inner)
+        orun(deck, steps=1, method=method, eps=args.eps, max_iters=1, inner_steps=args.inner)
     t_all, its, mv = 0.0, 0, 0
     for _ in range(args.steps):
         t0 = time.perf_counter()
-        _, st, _ = oracle.run(deck, steps=1, method=method, eps=args.eps,
-                              max_iters=sample_iters, inner_steps=args.inner)
+        _, st, _ = orun(deck, steps=1, method=method, eps=args.eps, max_iters=sample_iters,
+                        inner_steps=args.inner)
         t_all += time.perf_counter() - t0
         its += st[0]["iterations"]
         mv += st[0]["matvecs"]
@@ -179,20 +179,33 @@ METHOD_NAME = {"cppcg": "CPPCG", "cg": "CG", "bjcg": "block-Jacobi PCG",
                "cg1": "single-reduction CG", "jacobi": "Jacobi", "cheby": "Chebyshev"}
 
 
+def make_deck(args):
+    from paper_conf_cluster_mcintosh_smithm17_b200 import inputs
+    if args.nz > 1:
+        return inputs.crooked_pipe3(args.n, args.n, args.nz)
+    return inputs.crooked_pipe(args.n)
+
+
+def mesh_str(args):
+    return f"{args.n}x{args.n}" + (f"x{args.nz}" if args.nz > 1 else "")
+
+
 def metric_name(args):
-    return (f"solver iterations/s, {args.n}^2 {METHOD_NAME[args.method]}"
+    return (f"solver iterations/s, {mesh_str(args)} {METHOD_NAME[args.method]}"
             f" (time-to-solution, HBM GB/s alongside)")
 
 
 def config(args):
-    return {"workload": f"crooked_pipe {args.n}x{args.n} "
+    return {"workload": f"crooked_pipe{'3' if args.nz > 1 else ''} {mesh_str(args)} "
                         f"{'CPPCG s=' + str(args.inner) if args.method == 'cppcg' else METHOD_NAME[args.method]}"
                         f" eps={args.eps:g} 1 timestep/step",
-            "mesh": [args.n, args.n], "method": args.method, "inner_steps": args.inner,
+            "mesh": [args.n, args.n] + ([args.nz] if args.nz > 1 else []),
+            "method": args.method, "inner_steps": args.inner,
             "eps": args.eps, "max_iters": args.max_iters, "halo_depth": args.halo_depth,
             "dt": 0.004,
-            "l2": "inputs larger than L2 (12 fp64 fields x 134 MB at 4096^2)"
-            if args.n >= 2048 else "working set fits in L2 (no flush)"}
+            "l2": "inputs larger than L2 (>= 12 fp64 fields x 8 B x cells > 126 MB)"
+            if args.n * args.n * max(args.nz, 1) >= 2 ** 21 else
+            "working set fits in L2 (no flush)"}
 
 
 # ------------------------------------------------------------------ GPU arm
@@ -202,8 +215,9 @@ def cpu_baseline(args, deck):
     method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
               "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY}[args.method]
     t0 = time.perf_counter()
-    _, st, _ = oracle.run(deck, steps=1, method=method, eps=args.eps, max_iters=args.ref_iters,
-                          inner_steps=args.inner)
+    orun = oracle.run3 if args.nz > 1 else oracle.run
+    _, st, _ = orun(deck, steps=1, method=method, eps=args.eps, max_iters=args.ref_iters,
+                    inner_steps=args.inner)
     dt = time.perf_counter() - t0
     return {"value": st[0]["iterations"] / dt, "unit": "iterations/s", "cores": 1,
             "kind": "oracle",
@@ -263,10 +277,10 @@ def run_gpu(args):
         pg.all_reduce(t, op=pg.ReduceOp.MAX)
         return float(t.item())
 
-    deck = inputs.crooked_pipe(args.n)
+    deck = make_deck(args)
     method = {"cppcg": tea.CPPCG, "cg": tea.CG, "bjcg": tea.BJCG,
               "cg1": tea.CG1, "jacobi": tea.JACOBI, "cheby": tea.CHEBY}[args.method]
-    cells = args.n * args.n
+    cells = args.n * args.n * max(args.nz, 1)
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
                 tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode)
     stream = t.stream
@@ -310,7 +324,8 @@ def run_gpu(args):
         model_bytes = len(stats) * 5 * 8 * cells + iters * cg_iter_bytes(cells)
 
     # ---- e2e through the C ABI with host buffers (pinned)
-    u_host = torch.empty((args.n, args.n), dtype=torch.float64).pin_memory()
+    u_host = torch.empty(((args.nz,) if args.nz > 1 else ()) + (args.n, args.n),
+                         dtype=torch.float64).pin_memory()
     u_np = u_host.numpy()
     t.fetch(u_np)
     barrier()
@@ -391,6 +406,8 @@ def main():
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", default="b200", choices=["b200", "reference"])
     ap.add_argument("--n", type=int, default=4096)
+    ap.add_argument("--nz", type=int, default=0,
+                    help="> 1: the 3D 7-point problem on n x n x nz (SURVEY NEXT-4)")
     ap.add_argument("--method", default="cppcg", choices=["cppcg", "cg", "bjcg", "cg1", "jacobi", "cheby"])
     ap.add_argument("--inner", type=int, default=10)
     ap.add_argument("--eps", type=float, default=1e-12)

@@ -50,8 +50,8 @@ __device__ bool grid_reduce2(double v0, double v1, double *partials, unsigned *t
     __shared__ double sh[2][kWarps];
     __shared__ bool last;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    const int nblk = gridDim.x * gridDim.y;
-    const int bid = blockIdx.y * gridDim.x + blockIdx.x;
+    const int nblk = gridDim.x * gridDim.y * gridDim.z;
+    const int bid = (blockIdx.z * gridDim.y + blockIdx.y) * gridDim.x + blockIdx.x;
     v0 = wsum(v0);
     v1 = wsum(v1);
     if (lane == 0) {
@@ -97,7 +97,7 @@ __device__ bool grid_arrive2(unsigned *ticket) {
     __syncthreads();
     if (threadIdx.x == 0) {
         __threadfence();
-        last = (atomicAdd(ticket, 1u) == gridDim.x * gridDim.y - 1u);
+        last = (atomicAdd(ticket, 1u) == gridDim.x * gridDim.y * gridDim.z - 1u);
     }
     __syncthreads();
     if (last && threadIdx.x == 0) *ticket = 0u;
@@ -138,7 +138,7 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
 
     Scalars *S = a.S;
     if (S->done) {
-        if (LAST && blockIdx.x == 0 && blockIdx.y == 0 && threadIdx.x == 0 && a.set_cond &&
+        if (LAST && blockIdx.x == 0 && blockIdx.y == 0 && blockIdx.z == 0 && threadIdx.x == 0 && a.set_cond &&
             a.cond)
             cudaGraphSetConditional(a.cond, 0u);
         return;
@@ -300,7 +300,7 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
             }
         }
     } else if (FUSE) {
-        if (blockIdx.x == 0 && blockIdx.y == 0 && threadIdx.x == 0) S->alpha_prev = alpha;
+        if (blockIdx.x == 0 && blockIdx.y == 0 && blockIdx.z == 0 && threadIdx.x == 0) S->alpha_prev = alpha;
     }
 }
 

@@ -14,6 +14,8 @@ run --method cppcg --n 1024 --steps 10 --warmup 3
 run --method cg --n 1024 --steps 10 --warmup 3
 run --method cg --n 128 --steps 10 --warmup 3 --eps 1e-15
 run --method cppcg --n 128 --steps 10 --warmup 3 --eps 1e-15
+run --method cg --n 256 --nz 256 --steps 3 --warmup 3
+run --method cppcg --n 256 --nz 256 --steps 3 --warmup 3
 python - $OUT <<'PY'
 import json, sys
 for l in open(sys.argv[1]):
