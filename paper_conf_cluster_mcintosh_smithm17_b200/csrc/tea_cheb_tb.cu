@@ -116,7 +116,8 @@ template <int M>
 struct TbGeom {
     static constexpr int MR = (M + 1) & ~1;  // margin, even (double2 alignment)
     static constexpr int OW = kStrip - 2 * MR;  // output columns per warp strip
-    static constexpr int D = M + 2;             // delay-line depth (rows)
+    static constexpr int D = 8;  // delay-line depth (rows k-M-1..k fit for M <= 6); a power of
+                                 // two so slots are (head - t) & 7, not a division
 };
 
 #ifndef TEA_TB_MINB
@@ -132,9 +133,13 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
               int restart) {
     using G = TbGeom<M>;
     constexpr int D = G::D;
-    __shared__ double2 ringKx[D][kThreads], ringKy[D][kThreads], ringR[D][kThreads];
-    __shared__ double2 ringZ2[2][kThreads];
-    __shared__ double coef[4][M];
+    static_assert(M <= 6, "delay lines hold M+2 rows");
+    extern __shared__ double2 tb_smem[];
+    double2(*ringKx)[kThreads] = reinterpret_cast<double2(*)[kThreads]>(tb_smem);
+    double2(*ringKy)[kThreads] = ringKx + D;
+    double2(*ringR)[kThreads] = ringKy + D;
+    double2(*ringZ2)[kThreads] = ringR + D;
+    double(*coef)[M] = reinterpret_cast<double(*)[M]>(ringZ2 + 2);
 
     Scalars *S = a.S;
     if (S->done) {
@@ -191,11 +196,12 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
     for (int t = 0; t < M; ++t) W[t][0] = W[t][1] = W[t][2] = z0;
     double dot0 = 0.0, dot1 = 0.0;
 
-    // prefetch registers for input row k
+    // prefetch registers for input row k; running element offsets (no k*pitch products)
     double2 pX = z0, pW = z0, pZ2 = z0, pKx = z0, pKy = z0, pR = z0;
-    auto load = [&](int k) {
-        if (!ld_ok || kt0 >= kt1) return;
-        const int o = k * pitch + jA;
+    const int kbeg = kt0 - M, kend = kt1 + M;
+    long long orow = (long long)kbeg * pitch + jA;  // offset of (jA, k)
+    auto load = [&](long long o) {
+        if (!ld_ok) return;
         if (FIRST) {
             pX = ldg2c(rin + o);
             if (FUSE) pW = ldg2c(win + o);
@@ -207,71 +213,73 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
         pKx = ldg2c(Kx + o);
         pKy = ldg2c(Ky + o);
     };
-    const int kbeg = kt0 - M, kend = kt1 + M;
-    load(kbeg);
+    if (kt0 < kt1) load(orow);
+    int head = 0;  // ring slot of row k
 #pragma unroll(kTbUnroll)
-    for (int k = kbeg; k < kend; ++k) {
+    for (int k = kbeg; k < kend; ++k, orow += pitch, head = (head + 1) & (D - 1)) {
         double2 X = pX, Wv = pW, Z2 = pZ2, KX = pKx, KY = pKy, RR = pR;
-        if (k + 1 < kend) load(k + 1);
+        if (k + 1 < kend) load(orow + pitch);
         double2 rk;
         if (FIRST) {
             if (FUSE) X = make_double2(X.x - alpha * Wv.x, X.y - alpha * Wv.y);
             rk = X;
-            if (FUSE && k >= kt0 && k < kt1) st2m(rout + k * pitch + jA, X, oA, oB);
+            if (FUSE && k >= kt0 && k < kt1) st2m(rout + orow, X, oA, oB);
         } else {
             rk = RR;
         }
-        const int slot = (k + 4 * D) % D;
-        ringKx[slot][tid] = KX;
-        ringKy[slot][tid] = KY;
-        ringR[slot][tid] = rk;
-        if (!FIRST) ringZ2[(k + 4) & 1][tid] = Z2;
+        ringKx[head][tid] = KX;
+        ringKy[head][tid] = KY;
+        ringR[head][tid] = rk;
+        if (!FIRST) ringZ2[k & 1][tid] = Z2;
         W[0][0] = W[0][1];
         W[0][1] = W[0][2];
         W[0][2] = X;
 #pragma unroll
         for (int t = 1; t <= M; ++t) {
             const int q = k - t;
-            const int sq = (q + 4 * D) % D, sq1 = (q + 1 + 4 * D) % D;
+            const int sq = (head - t) & (D - 1), sq1 = (head - t + 1) & (D - 1);
             const double2 kx = ringKx[sq][tid];
             const double2 kyc = ringKy[sq][tid];
             const double2 kyn = ringKy[sq1][tid];
             const double2 rq = ringR[sq][tid];
             double2 z2;
             if (t == 1) {
-                z2 = FIRST ? z0 : ringZ2[(q + 4) & 1][tid];
+                z2 = FIRST ? z0 : ringZ2[(k + 1) & 1][tid];  // row k-1
             } else {
                 z2 = W[t >= 2 ? t - 2 : 0][0];
             }
             const double2 xm = W[t - 1][0], xc = W[t - 1][1], xp = W[t - 1][2];
-            double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
-            double right = __shfl_down_sync(0xffffffffu, xc.x, 1);
-            double kxB = __shfl_down_sync(0xffffffffu, kx.x, 1);
-            if (lane == 0) left = 0.0;
-            if (lane == 31) {
-                right = 0.0;
-                kxB = 0.0;
-            }
-            double2 AX;
-            AX.x = (1.0 + (kyn.x + kyc.x) + (kx.y + kx.x)) * xc.x - (kyn.x * xp.x + kyc.x * xm.x) -
-                   (kx.y * xc.y + kx.x * left);
-            AX.y = (1.0 + (kyn.y + kyc.y) + (kxB + kx.y)) * xc.y - (kyn.y * xp.y + kyc.y * xm.y) -
-                   (kxB * right + kx.y * xc.x);
+            // lane 0's left and lane 31's right neighbours are outside the strip: the
+            // shuffles return the lane's own (finite) value, which only pollutes the
+            // overlap columns every step already discards -- no selects needed
+            const double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
+            const double right = __shfl_down_sync(0xffffffffu, xc.x, 1);
+            const double kxB = __shfl_down_sync(0xffffffffu, kx.x, 1);
+            // Dependency order: xp (the "up" row) is the row step t-1 produced in THIS
+            // row-iteration; everything else is older. Form the rest first, fold xp in
+            // last (A x = Listing 1; only the rounding order of the sums differs).
             const double cx = coef[0][t - 1], cz = coef[1][t - 1], cr = coef[2][t - 1],
                          ca = coef[3][t - 1];
+            double2 AXo, base;  // A x without the up term; the step's x-independent part
+            AXo.x = (1.0 + (kyn.x + kyc.x) + (kx.y + kx.x)) * xc.x - kyc.x * xm.x -
+                    (kx.y * xc.y + kx.x * left);
+            AXo.y = (1.0 + (kyn.y + kyc.y) + (kxB + kx.y)) * xc.y - kyc.y * xm.y -
+                    (kxB * right + kx.y * xc.x);
+            base.x = cx * xc.x + cz * z2.x + cr * rq.x;
+            base.y = cx * xc.y + cz * z2.y + cr * rq.y;
             double2 zn;
-            zn.x = cx * xc.x + cz * z2.x + cr * rq.x - ca * AX.x;
-            zn.y = cx * xc.y + cz * z2.y + cr * rq.y - ca * AX.y;
+            zn.x = fma(-ca, fma(-kyn.x, xp.x, AXo.x), base.x);
+            zn.y = fma(-ca, fma(-kyn.y, xp.y, AXo.y), base.y);
             const bool rowout = q >= kt0 && q < kt1;
             if (t < M) {
                 const int tt = t < M ? t : M - 1;
                 W[tt][0] = W[tt][1];
                 W[tt][1] = W[tt][2];
                 W[tt][2] = zn;
-                if (t == M - 1 && !LAST && rowout) st2m(zoutA + q * pitch + jA, zn, oA, oB);
+                if (t == M - 1 && !LAST && rowout) st2m(zoutA + (orow - t * pitch), zn, oA, oB);
             } else {
                 if (rowout) {
-                    st2m(zoutB + q * pitch + jA, zn, oA, oB);
+                    st2m(zoutB + (orow - t * pitch), zn, oA, oB);
                     if (LAST) {
                         if (oA) {
                             dot0 += rq.x * zn.x;
@@ -318,7 +326,15 @@ static void tb_launch(const KArgs &a, const Region &R, int ty, int jlim, int ste
     const int width = R.j1;  // single block: R.j0 == 0
     const int nstrips = (width + G::OW - 1) / G::OW;
     dim3 grid((nstrips + kWarps - 1) / kWarps, (R.k1 - R.k0 + ty - 1) / ty);
-    k_cheb_tb<M, FIRST, FUSE, LAST><<<grid, kThreads, 0, st>>>(
+    constexpr size_t smem =
+        sizeof(double2) * (3 * G::D + 2) * kThreads + sizeof(double) * 4 * M;
+    static bool attr = false;  // per instantiation
+    if (!attr) {
+        cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST>,
+                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        attr = true;
+    }
+    k_cheb_tb<M, FIRST, FUSE, LAST><<<grid, kThreads, smem, st>>>(
         rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, a, R, ty, jlim, step0, restart ? 1 : 0);
 }
 
