@@ -123,6 +123,10 @@ struct TbGeom {
 #ifndef TEA_TB_MINB
 #define TEA_TB_MINB 1
 #endif
+#ifndef TEA_TB_REGLINES
+#define TEA_TB_REGLINES 0  // 1: register shift registers (measured slower: 225 regs,
+                            // 2 CTAs/SM, 737 vs 660 us/outer, profiles/r01_tb_reglines.txt)
+#endif
 template <int M, bool FIRST, bool FUSE, bool LAST>
 __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
     k_cheb_tb(const double *__restrict__ rin, const double *__restrict__ win,
@@ -215,6 +219,11 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
     };
     if (kt0 < kt1) load(orow);
     int head = 0;  // ring slot of row k
+#if TEA_TB_REGLINES
+    double2 rKx[M + 1], rKy[M + 1], rR[M + 1], z2prev = z0;
+#pragma unroll
+    for (int i = 0; i <= M; ++i) rKx[i] = rKy[i] = rR[i] = z0;
+#endif
 #pragma unroll(kTbUnroll)
     for (int k = kbeg; k < kend; ++k, orow += pitch, head = (head + 1) & (D - 1)) {
         double2 X = pX, Wv = pW, Z2 = pZ2, KX = pKx, KY = pKy, RR = pR;
@@ -227,16 +236,42 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
         } else {
             rk = RR;
         }
+#if TEA_TB_REGLINES
+        // delay lines as register shift registers: index i holds row k - i (the step
+        // loop is unrolled, so step t's lag t is a compile-time index) -- register moves
+        // on the ALU pipes instead of shared-memory wavefronts through L1TEX
+#pragma unroll
+        for (int i = M; i > 0; --i) {
+            rKx[i] = rKx[i - 1];
+            rKy[i] = rKy[i - 1];
+            rR[i] = rR[i - 1];
+        }
+        rKx[0] = KX;
+        rKy[0] = KY;
+        rR[0] = rk;
+        const double2 z2row = z2prev;  // z_{i-2} of row k-1
+        if (!FIRST) z2prev = Z2;
+#else
         ringKx[head][tid] = KX;
         ringKy[head][tid] = KY;
         ringR[head][tid] = rk;
         if (!FIRST) ringZ2[k & 1][tid] = Z2;
+#endif
         W[0][0] = W[0][1];
         W[0][1] = W[0][2];
         W[0][2] = X;
 #pragma unroll
         for (int t = 1; t <= M; ++t) {
             const int q = k - t;
+#if TEA_TB_REGLINES
+            const double2 kx = rKx[t], kyc = rKy[t], kyn = rKy[t - 1], rq = rR[t];
+            double2 z2;
+            if (t == 1) {
+                z2 = FIRST ? z0 : z2row;
+            } else {
+                z2 = W[t >= 2 ? t - 2 : 0][0];
+            }
+#else
             const int sq = (head - t) & (D - 1), sq1 = (head - t + 1) & (D - 1);
             const double2 kx = ringKx[sq][tid];
             const double2 kyc = ringKy[sq][tid];
@@ -248,6 +283,7 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
             } else {
                 z2 = W[t >= 2 ? t - 2 : 0][0];
             }
+#endif
             const double2 xm = W[t - 1][0], xc = W[t - 1][1], xp = W[t - 1][2];
             // lane 0's left and lane 31's right neighbours are outside the strip: the
             // shuffles return the lane's own (finite) value, which only pollutes the
