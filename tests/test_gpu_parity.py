@@ -467,3 +467,15 @@ def test_3d_rejections(tea):
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt)
     assert t.solve(method=2, raise_on_error=False).status == tea.ERR_ARG  # block Jacobi: 2D
     t.close()
+
+
+@pytest.mark.parametrize("loop_mode", [1, 2])
+def test_loop_modes_identical_fused_passes(tea, loop_mode):
+    """The WHILE graph, chunked graphs and eager launches agree bitwise on a mesh large
+    enough for the fused Chebyshev passes (>= 2M cells)."""
+    deck = deck_of("pipe", 2048, 1100)
+    kw = dict(method=1, eps=1e-10, max_iters=2000, inner_steps=10)
+    ref, st_ref = gpu_run(tea, deck, loop_mode=0, **kw)
+    u, st = gpu_run(tea, deck, loop_mode=loop_mode, check_interval=6, **kw)
+    assert st[0]["iterations"] == st_ref[0]["iterations"]
+    assert np.array_equal(u, ref)
