@@ -479,3 +479,22 @@ def test_loop_modes_identical_fused_passes(tea, loop_mode):
     u, st = gpu_run(tea, deck, loop_mode=loop_mode, check_interval=6, **kw)
     assert st[0]["iterations"] == st_ref[0]["iterations"]
     assert np.array_equal(u, ref)
+
+
+# ---------------------------------------------------------------- sanitizers
+@pytest.mark.parametrize("tool", ["memcheck", "racecheck"])
+def test_compute_sanitizer(tea, tool):
+    """compute-sanitizer over small solves of every path (tools/sanitize.py): no memory
+    errors, no shared-memory races (the fused passes' delay lines, the grid reductions)."""
+    import shutil
+    import subprocess
+    import sys
+    exe = shutil.which("compute-sanitizer") or "/usr/local/cuda/bin/compute-sanitizer"
+    if not os.path.exists(exe):
+        pytest.skip("compute-sanitizer not found")
+    root = os.path.dirname(HERE)
+    out = subprocess.run([exe, "--tool", tool, "--error-exitcode", "9", sys.executable,
+                          os.path.join(root, "tools", "sanitize.py")], capture_output=True,
+                         text=True, timeout=900, cwd=root)
+    assert out.returncode == 0, out.stdout[-3000:] + out.stderr[-3000:]
+    assert "0 errors" in out.stdout or "0 hazards" in out.stdout

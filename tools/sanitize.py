@@ -1,0 +1,34 @@
+"""Small solves of every path, for compute-sanitizer (memcheck / racecheck / synccheck /
+initcheck). Eager launches (loop mode 2) so every kernel is visible to the tool.
+
+compute-sanitizer --tool memcheck --error-exitcode 9 python tools/sanitize.py
+"""
+import os
+import sys
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+
+
+def main():
+    import paper_conf_cluster_mcintosh_smithm17_b200 as tea
+    from paper_conf_cluster_mcintosh_smithm17_b200 import inputs
+    cases = [
+        (inputs.crooked_pipe(96, 70), None, dict(tb_steps=1)),
+        (inputs.crooked_pipe(96, 70), None, dict(tb_steps=5)),      # fused passes forced on
+        (inputs.random_fields(67, 45, 3), dict(px=2, py=2, halo_depth=3, nranks=1), {}),
+        (inputs.crooked_pipe3(20, 18, 9), None, {}),
+    ]
+    for deck, dist, kw in cases:
+        for method in (0, 1, 2, 3, 4, 5):
+            if getattr(deck, "nz", 1) > 1 and method == 2:
+                continue
+            t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist,
+                        loop_mode=2, check_interval=4, presteps=10, **kw)
+            r = t.solve(method, 1e-10, 60, 4, raise_on_error=False)
+            t.fetch()
+            t.close()
+            print(deck.name, dist, kw, method, r.status, r.stats["iterations"], flush=True)
+
+
+if __name__ == "__main__":
+    main()
