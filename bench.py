@@ -277,6 +277,9 @@ def run_gpu(args):
         pg.all_reduce(t, op=pg.ReduceOp.MAX)
         return float(t.item())
 
+    if args.blocks and world == 1:
+        bpx, bpy = (int(v) for v in args.blocks.lower().split("x"))
+        dist_kw = dict(rank=0, nranks=1, px=bpx, py=bpy, halo_depth=args.halo_depth)
     deck = make_deck(args)
     method = {"cppcg": tea.CPPCG, "cg": tea.CG, "bjcg": tea.BJCG,
               "cg1": tea.CG1, "jacobi": tea.JACOBI, "cheby": tea.CHEBY}[args.method]
@@ -337,7 +340,7 @@ def run_gpu(args):
         t.fetch(u_np)
     torch.cuda.synchronize()
     e_dt = max_over_ranks(time.perf_counter() - e0)
-    bx = cells // world
+    bx = cells // world  # host bytes this rank copies per step
     e2e = {"value": e_iters / e_dt, "unit": "iterations/s", "h2d_bytes_per_step": 8 * bx,
            "d2h_bytes_per_step": 8 * bx}
     t.close()
@@ -375,8 +378,10 @@ def run_gpu(args):
         "n_gpus": world, "steps": args.steps, "warmup": args.warmup,
         "ms_per_step": ms / args.steps, "higher_is_better": True, "scaling": "strong",
         "vs_baseline": None, "dtype": "f64", "data": "synthetic (crooked pipe deck, seeded)",
-        "config": dict(config(args), parallelism=f"{dist_kw['px']}x{dist_kw['py']} blocks"
-                       if dist_kw else "1 block"),
+        "config": dict(config(args), parallelism=(
+            f"{dist_kw['px']}x{dist_kw['py']} blocks" +
+            (" in one process (device-copy halos)" if dist_kw and world == 1 else "")
+            if dist_kw else "1 block")),
         "time_to_solution_s": ms * 1e-3 / args.steps,
         "iterations_per_step": iters / args.steps, "outer_per_step": outer / args.steps,
         "matvecs_per_s": matvecs / (ms * 1e-3),
@@ -415,6 +420,9 @@ def main():
                     help="0 = 100000 (Krylov methods) or 2000 (jacobi/cheby: a fixed-work "
                          "throughput run; they need O(kappa) iterations at 4096^2)")
     ap.add_argument("--halo-depth", type=int, default=2)
+    ap.add_argument("--blocks", default="",
+                    help="PXxPY: run the px x py decomposition inside ONE process on one GPU "
+                         "(the multi-GPU code path with device-copy halos instead of NCCL)")
     ap.add_argument("--tile-rows", type=int, default=0)
     ap.add_argument("--tb-steps", type=int, default=0,
                     help="Chebyshev steps per fused HBM pass (0 auto=4, 1 = per-step kernels)")

@@ -15,6 +15,10 @@ run --method cg --n 1024 --steps 10 --warmup 3
 run --method cg --n 128 --steps 10 --warmup 3 --eps 1e-15
 run --method cppcg --n 128 --steps 10 --warmup 3 --eps 1e-15
 run --method cg --n 256 --nz 256 --steps 3 --warmup 3
+run --method cppcg --n 4096 --steps 3 --warmup 3 --blocks 2x4 --halo-depth 2
+run --method cppcg --n 4096 --steps 3 --warmup 3 --blocks 2x4 --halo-depth 10
+run --method cg --n 4096 --steps 3 --warmup 3 --blocks 2x4 --halo-depth 1
+run --method cppcg --n 16384 --steps 1 --warmup 3 --max-iters 100000
 run --method cppcg --n 256 --nz 256 --steps 3 --warmup 3
 python - $OUT <<'PY'
 import json, sys
