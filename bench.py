@@ -419,7 +419,9 @@ def main():
     ap.add_argument("--max-iters", type=int, default=0,
                     help="0 = 100000 (Krylov methods) or 2000 (jacobi/cheby: a fixed-work "
                          "throughput run; they need O(kappa) iterations at 4096^2)")
-    ap.add_argument("--halo-depth", type=int, default=2)
+    ap.add_argument("--halo-depth", type=int, default=0,
+                    help="0 = auto: inner+1 for CPPCG (one deep exchange per outer, fused "
+                         "passes on extended bounds), 1 otherwise")
     ap.add_argument("--blocks", default="",
                     help="PXxPY: run the px x py decomposition inside ONE process on one GPU "
                          "(the multi-GPU code path with device-copy halos instead of NCCL)")
@@ -433,6 +435,8 @@ def main():
     args = ap.parse_args()
     if args.warmup < 3:
         ap.error("--warmup must be >= 3")
+    if args.halo_depth == 0:
+        args.halo_depth = args.inner + 1 if args.method == "cppcg" else 1
     if args.max_iters == 0:
         args.max_iters = 2000 if args.method in ("jacobi", "cheby") else 100000
     if args.impl == "reference":

@@ -66,9 +66,11 @@ BlockLayout layout_block(const tea_mesh &m, int px, int py, int d, int b) {
     split(m.ny, py, L.bj, &L.gy0, &L.gy1);
     L.bx = L.gx1 - L.gx0;
     L.by = L.gy1 - L.gy0;
-    L.H = std::max(d + 2, kTbMaxSteps + 2);  // the fused passes read M rows past a tile
-    L.X0 = (int)round_up(d + 4, 16);
-    L.pitch = (int)round_up(L.X0 + L.bx + d + 4, 32);
+    // halo margins: the fused passes read up to M (<= 5) rows and MR (<= 6) columns beyond
+    // their output region, which reaches d cells into the halo on extended bounds
+    L.H = d + kTbMaxSteps + 2;
+    L.X0 = (int)round_up(d + 8, 16);
+    L.pitch = (int)round_up(L.X0 + L.bx + d + 8, 32);
     L.rows = L.by + 2 * L.H;
     L.nz = m.nz > 1 ? m.nz : 1;
     L.ps = (long long)L.rows * L.pitch;
@@ -533,61 +535,78 @@ int tb_steps(const tea_ctx *c) {
     return std::min(m, kTbMaxSteps);
 }
 
-// Temporally blocked chain (single block): passes of M steps, each ONE kernel
+bool single_block(tea_ctx *c) { return c->px * c->py == 1; }
+bool is3d(const tea_ctx *c) { return c->blocks[0].L.nz > 1; }
+
+// Temporally blocked chain: passes of M steps, each ONE kernel per block
 // (tea_cheb_tb.cu). z pairs ping-pong: pass p writes (z_{last-1}, z_last) into
 // pair p%2 = (Z0,Z1) or (Z2,Z3). Returns the field holding z_s.
+// With neighbour blocks (matrix powers, P:L423-495 -- on chip): r is exchanged ONCE at
+// depth d >= s + 1 (corners included); pass p then runs on bounds extended by
+// 1 + (steps after it), so the last pass leaves z_s valid on the 1-cell ring the next
+// SpMV reads; no z exchange. (One block: every extension is empty.)
 int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout,
                   bool sets_cond) {
     const auto passes = tb_passes(s, tb_steps(c));
     const int pairA[2] = {F_Z0, F_Z2}, pairB[2] = {F_Z1, F_Z3};
-    BlockCtx &b = c->blocks[0];
-    const Region R = b.owned();
-    const int jlim = b.L.pitch - b.L.X0;
-    int step0 = 1;
+    const bool blocks = !single_block(c);
+    if (blocks) exchange(c, X_RD, {rin});  // depth d >= s + 1, with corners
+    int step0 = 1, after = s;
     const int r = fused ? rout : rin;
     for (size_t p = 0; p < passes.size(); ++p) {
         const int M = passes[p];
+        after -= M;
         const bool first = p == 0, last = p + 1 == passes.size();
         const bool fu = fused && first;
         const int o = p % 2, in = (p + 1) % 2;
-        int ty = c->opts.tb_rows > 0 ? c->opts.tb_rows : 0;
-        if (ty <= 0) {
-            // tall tiles keep the 2M-row pipeline fill small; enough CTAs for ~2 waves
-            // at 3 CTAs/SM. Measured at 4096^2, M = 5 (profiles/r01_tb_rows.txt):
-            // 96 rows 667 us/outer, 64 rows 688, 32 rows 754.
-            const int cand[] = {96, 64, 32, 16};
-            for (int cnd : cand) {
-                ty = cnd;
-                if (tb_ctas(M, R.j1, R.k1, ty) >= 800) break;
+        for (auto &b : c->blocks) {
+            const Region R = blocks ? b.ext(1 + after) : b.owned();
+            const Region D = b.owned();
+            const int jlim = b.L.pitch - b.L.X0;
+            int ty = c->opts.tb_rows > 0 ? c->opts.tb_rows : 0;
+            if (ty <= 0) {
+                // tall tiles keep the 2M-row pipeline fill small; enough CTAs for ~2
+                // waves at 3 CTAs/SM. Measured at 4096^2, M = 5 (r01_tb_rows.txt):
+                // 96 rows 667 us/outer, 64 rows 688, 32 rows 754.
+                const int cand[] = {96, 64, 32, 16};
+                for (int cnd : cand) {
+                    ty = cnd;
+                    if (tb_ctas(M, R.j1 - R.j0, R.k1 - R.k0, ty) >= 800) break;
+                }
             }
+            int streams = first ? (fu ? 4 : 3) : 5;     // reads
+            streams += (fu ? 1 : 0) + (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})
+            const int kid = last ? TEA_K_TB_LAST : (first ? TEA_K_TB_FIRST : TEA_K_TB_MID);
+            K(c, kid, sbytes(b, streams), [&] {
+                launch_cheb_tb(kargs(c, b, last && sets_cond), R, D, M, ty, jlim, step0, first,
+                               fu, last, restart, b.f[first && fu ? rin : r], b.f[F_W],
+                               b.f[rout], first ? nullptr : b.f[pairB[in]],
+                               first ? nullptr : b.f[pairA[in]], b.f[pairA[o]], b.f[pairB[o]],
+                               b.f[F_KX], b.f[F_KY], c->stream);
+            });
         }
-        int streams = first ? (fu ? 4 : 3) : 5;     // reads
-        streams += (fu ? 1 : 0) + (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})
-        const int kid = last ? TEA_K_TB_LAST : (first ? TEA_K_TB_FIRST : TEA_K_TB_MID);
-        K(c, kid, sbytes(b, streams), [&] {
-            launch_cheb_tb(kargs(c, b, last && sets_cond), R, M, ty, jlim, step0, first, fu,
-                           last, restart, b.f[first && fu ? rin : r], b.f[F_W], b.f[rout],
-                           first ? nullptr : b.f[pairB[in]], first ? nullptr : b.f[pairA[in]],
-                           b.f[pairA[o]], b.f[pairB[o]], b.f[F_KX], b.f[F_KY], c->stream);
-        });
         step0 += M;
     }
     reduce(c, 1, 2);
     return pairB[(passes.size() - 1) % 2];
 }
 
-bool single_block(tea_ctx *c) { return c->px * c->py == 1; }
-bool is3d(const tea_ctx *c) { return c->blocks[0].L.nz > 1; }
+
+// fused passes: 2D; with neighbour blocks only when the halo is deep enough for the whole
+// chain at once (d >= s + 1, the paper's deep-halo regime)
+bool use_tb(tea_ctx *c, int s) {
+    if (is3d(c) || tb_steps(c) <= 1) return false;
+    return single_block(c) || c->d >= s + 1;
+}
 
 int chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond) {
-    if (single_block(c) && !is3d(c) && tb_steps(c) > 1)
-        return cheb_chain_tb(c, s, restart, fused, rin, rout, sets_cond);
+    if (use_tb(c, s)) return cheb_chain_tb(c, s, restart, fused, rin, rout, sets_cond);
     return cheb_chain(c, s, restart, fused, rin, rout, sets_cond);
 }
 
 // field holding z_s after a chain (same for every chain of a context and s)
 int zs_field(tea_ctx *c, int s) {
-    if (single_block(c) && !is3d(c) && tb_steps(c) > 1) {
+    if (use_tb(c, s)) {
         const int P = (int)tb_passes(s, tb_steps(c)).size();
         return (P - 1) % 2 == 0 ? F_Z1 : F_Z3;
     }

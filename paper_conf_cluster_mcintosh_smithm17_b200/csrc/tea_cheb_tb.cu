@@ -133,8 +133,8 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
               double *__restrict__ rout, const double *__restrict__ zin1,
               const double *__restrict__ zin2, double *__restrict__ zoutA,
               double *__restrict__ zoutB, const double *__restrict__ Kx,
-              const double *__restrict__ Ky, KArgs a, Region R, int ty, int jlim, int step0,
-              int restart) {
+              const double *__restrict__ Ky, KArgs a, Region R, Region Dd, int ty, int jlim,
+              int step0, int restart) {
     using G = TbGeom<M>;
     constexpr int D = G::D;
     static_assert(M <= 6, "delay lines hold M+2 rows");
@@ -184,7 +184,9 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
 
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5, tid = threadIdx.x;
     const int strip = blockIdx.x * kWarps + warp;
-    const int jA = -G::MR + strip * G::OW + 2 * lane;
+    // strips tile the output region R (which may reach into the halo on sides with a
+    // neighbour block: extended bounds); first strip starts MR before it
+    const int jA = (R.j0 & ~1) - G::MR + strip * G::OW + 2 * lane;
     const int kt0 = R.k0 + blockIdx.y * ty;
     const int kt1 = min(kt0 + ty, R.k1);
     const int pitch = a.pitch;
@@ -193,6 +195,8 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
     const int cA = 2 * lane, cB = 2 * lane + 1;
     const bool oA = cA >= G::MR && cA < kStrip - G::MR && jA >= R.j0 && jA < R.j1;
     const bool oB = cB >= G::MR && cB < kStrip - G::MR && jA + 1 >= R.j0 && jA + 1 < R.j1;
+    // dot products over owned cells only (D), whatever the extension of R
+    const bool dA = oA && jA >= Dd.j0 && jA < Dd.j1, dB = oB && jA + 1 >= Dd.j0 && jA + 1 < Dd.j1;
 
     // stencil windows: W[t] holds z_t rows (oldest, middle, newest); W[0] = input operand
     double2 W[M][3];
@@ -316,12 +320,12 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
             } else {
                 if (rowout) {
                     st2m(zoutB + (orow - t * pitch), zn, oA, oB);
-                    if (LAST) {
-                        if (oA) {
+                    if (LAST && q >= Dd.k0 && q < Dd.k1) {
+                        if (dA) {
                             dot0 += rq.x * zn.x;
                             dot1 += rq.x * rq.x;
                         }
-                        if (oB) {
+                        if (dB) {
                             dot0 += rq.y * zn.y;
                             dot1 += rq.y * rq.y;
                         }
@@ -354,12 +358,13 @@ int tb_out_cols(int M) {
 }
 
 template <int M, bool FIRST, bool FUSE, bool LAST>
-static void tb_launch(const KArgs &a, const Region &R, int ty, int jlim, int step0, bool restart,
+static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty, int jlim,
+                      int step0, bool restart,
                       const double *rin, const double *win, double *rout, const double *zin1,
                       const double *zin2, double *zoutA, double *zoutB, const double *kx,
                       const double *ky, cudaStream_t st) {
     using G = TbGeom<M>;
-    const int width = R.j1;  // single block: R.j0 == 0
+    const int width = R.j1 - (R.j0 & ~1);
     const int nstrips = (width + G::OW - 1) / G::OW;
     dim3 grid((nstrips + kWarps - 1) / kWarps, (R.k1 - R.k0 + ty - 1) / ty);
     constexpr size_t smem =
@@ -371,16 +376,17 @@ static void tb_launch(const KArgs &a, const Region &R, int ty, int jlim, int ste
         attr = true;
     }
     k_cheb_tb<M, FIRST, FUSE, LAST><<<grid, kThreads, smem, st>>>(
-        rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, a, R, ty, jlim, step0, restart ? 1 : 0);
+        rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, a, R, Dd, ty, jlim, step0, restart ? 1 : 0);
 }
 
 template <int M>
-static void tb_dispatch(const KArgs &a, const Region &R, int ty, int jlim, int step0, bool first,
+static void tb_dispatch(const KArgs &a, const Region &R, const Region &Dd, int ty, int jlim,
+                        int step0, bool first,
                         bool fuse, bool last, bool restart, const double *rin, const double *win,
                         double *rout, const double *zin1, const double *zin2, double *zoutA,
                         double *zoutB, const double *kx, const double *ky, cudaStream_t st) {
 #define TB(F, U, L)                                                                            \
-    tb_launch<M, F, U, L>(a, R, ty, jlim, step0, restart, rin, win, rout, zin1, zin2, zoutA, \
+    tb_launch<M, F, U, L>(a, R, Dd, ty, jlim, step0, restart, rin, win, rout, zin1, zin2, zoutA, \
                           zoutB, kx, ky, st)
     if (first) {
         if (fuse) {
@@ -402,17 +408,18 @@ int tb_ctas(int M, int width, int height, int ty) {
     return ((nstrips + kWarps - 1) / kWarps) * ((height + ty - 1) / ty);
 }
 
-void launch_cheb_tb(const KArgs &a, const Region &R, int M, int ty, int jlim, int step0,
+void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, int ty, int jlim,
+                    int step0,
                     bool first, bool fuse, bool last, bool restart, const double *rin,
                     const double *win, double *rout, const double *zin1, const double *zin2,
                     double *zoutA, double *zoutB, const double *kx, const double *ky,
                     cudaStream_t st) {
     switch (M) {
-        case 1: tb_dispatch<1>(a, R, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
-        case 2: tb_dispatch<2>(a, R, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
-        case 3: tb_dispatch<3>(a, R, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
-        case 4: tb_dispatch<4>(a, R, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
-        default: tb_dispatch<5>(a, R, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
+        case 1: tb_dispatch<1>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
+        case 2: tb_dispatch<2>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
+        case 3: tb_dispatch<3>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
+        case 4: tb_dispatch<4>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
+        default: tb_dispatch<5>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
     }
 }
 

@@ -158,8 +158,8 @@ void launch_cg1_w(const KArgs &a, const Launch &L, const Region &R, const double
 constexpr int kTbMaxSteps = 5;
 int tb_out_cols(int M);
 int tb_ctas(int M, int width, int height, int ty);
-void launch_cheb_tb(const KArgs &a, const Region &R, int M, int ty, int jlim, int step0,
-                    bool first, bool fuse, bool last, bool restart, const double *rin,
+void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, int ty, int jlim,
+                    int step0, bool first, bool fuse, bool last, bool restart, const double *rin,
                     const double *win, double *rout, const double *zin1, const double *zin2,
                     double *zoutA, double *zoutB, const double *kx, const double *ky,
                     cudaStream_t st);

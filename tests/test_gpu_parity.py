@@ -498,3 +498,31 @@ def test_compute_sanitizer(tea, tool):
                          text=True, timeout=900, cwd=root)
     assert out.returncode == 0, out.stdout[-3000:] + out.stderr[-3000:]
     assert "0 errors" in out.stdout or "0 hazards" in out.stdout
+
+
+# ---------------------------------------------------------------- fused passes on blocks
+@pytest.mark.parametrize("px,py,d,s,tb", [(2, 2, 11, 10, 5), (3, 2, 12, 10, 4), (2, 1, 16, 10, 5),
+                                          (1, 3, 6, 5, 3), (4, 2, 4, 3, 2), (2, 2, 11, 10, 1)])
+def test_fused_passes_on_extended_bounds(tea, ora, px, py, d, s, tb):
+    """Matrix powers on chip across blocks: one depth-d exchange of r per
+    outer iteration, fused passes on bounds extended by 1 + (steps after the pass)."""
+    deck = deck_of("pipe", 240, 200)
+    kw = dict(method=1, eps=1e-13, max_iters=20000, inner_steps=s)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, dist=dict(px=px, py=py, halo_depth=d, nranks=1),
+                        tb_steps=tb, **kw)
+    assert st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+    u_1, _ = gpu_run(tea, deck, tb_steps=tb, **kw)
+    assert rel_err(u_g, u_1) <= 1e-10
+
+
+def test_fused_passes_blocks_fixed_iterations(tea, ora):
+    deck = deck_of("random", 200, 150, seed=12, dt=0.04)
+    kw = dict(method=1, eps=0.0, max_iters=34, inner_steps=10)
+    u_o, _, _ = ora.run(deck, steps=1, **kw)
+    u_g, st = gpu_run(tea, deck, dist=dict(px=3, py=2, halo_depth=11, nranks=1), tb_steps=5,
+                      **kw)
+    assert st[0]["iterations"] == 34
+    assert field_err(u_g, u_o, "random") <= 1e-12
