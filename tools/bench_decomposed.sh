@@ -2,8 +2,12 @@ OUT=gpurun_out/bench_new.jsonl; : > $OUT
 run() { timeout 900 python bench.py "$@" --no-cpu 2>gpurun_out/bench_new_err.log | tail -1 >> $OUT; }
 run --method cppcg --n 4096 --steps 3 --warmup 3 --blocks 2x4 --halo-depth 2
 run --method cppcg --n 4096 --steps 3 --warmup 3 --blocks 2x4 --halo-depth 10
+run --method cppcg --n 4096 --steps 3 --warmup 3 --blocks 2x4 --halo-depth 11
+run --method cppcg --n 4096 --steps 3 --warmup 3 --blocks 2x4 --halo-depth 16
+run --method cppcg --n 4096 --steps 3 --warmup 3 --blocks 1x2 --halo-depth 11
+run --method cppcg --n 4096 --steps 3 --warmup 3 --blocks 2x2 --halo-depth 11
 run --method cg --n 4096 --steps 3 --warmup 3 --blocks 2x4 --halo-depth 1
-run --method cppcg --n 16384 --steps 1 --warmup 3
+run --method cppcg --n 16384 --steps 1 --warmup 3 --blocks 2x4 --halo-depth 11
 python - $OUT <<'PY'
 import json, sys
 for l in open(sys.argv[1]):
