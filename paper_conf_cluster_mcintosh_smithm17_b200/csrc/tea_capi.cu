@@ -145,6 +145,7 @@ struct tea_ctx {
     // capture state
     cudaGraphConditionalHandle cond = 0;
     int ty_override = 0;
+    int coef_slot = -1;  // constant-memory coefficient slot of the fused passes
 };
 
 static std::string g_init_error;
@@ -190,6 +191,7 @@ KArgs kargs(tea_ctx *c, const BlockCtx &b, bool set_cond = false) {
     a.kz = b.f[F_KZ];
     a.ps = b.L.ps;
     a.nz = b.L.nz;
+    a.coef_slot = c->coef_slot;
     return a;
 }
 
@@ -564,16 +566,8 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
             const Region D = b.owned();
             const int jlim = b.L.pitch - b.L.X0;
             int ty = c->opts.tb_rows > 0 ? c->opts.tb_rows : 0;
-            if (ty <= 0) {
-                // tall tiles keep the 2M-row pipeline fill small; enough CTAs for ~2
-                // waves at 3 CTAs/SM. Measured at 4096^2, M = 5 (r01_tb_rows.txt):
-                // 96 rows 667 us/outer, 64 rows 688, 32 rows 754.
-                const int cand[] = {96, 64, 32, 16};
-                for (int cnd : cand) {
-                    ty = cnd;
-                    if (tb_ctas(M, R.j1 - R.j0, R.k1 - R.k0, ty) >= 800) break;
-                }
-            }
+            // tall tiles keep the 2M-row pipeline fill small; whole waves (tb_auto_rows)
+            if (ty <= 0) ty = tb_auto_rows(M, R.j1 - R.j0, R.k1 - R.k0);
             int streams = first ? (fu ? 4 : 3) : 5;     // reads
             streams += (fu ? 1 : 0) + (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})
             const int kid = last ? TEA_K_TB_LAST : (first ? TEA_K_TB_FIRST : TEA_K_TB_MID);
@@ -595,7 +589,7 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
 // fused passes: 2D; with neighbour blocks only when the halo is deep enough for the whole
 // chain at once (d >= s + 1, the paper's deep-halo regime)
 bool use_tb(tea_ctx *c, int s) {
-    if (is3d(c) || tb_steps(c) <= 1) return false;
+    if (is3d(c) || tb_steps(c) <= 1 || c->coef_slot < 0) return false;
     return single_block(c) || c->d >= s + 1;
 }
 
@@ -910,6 +904,9 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         // ---- eigen-estimate, coefficients, restart z = B(A) r, p = z
         for (auto &b : c->blocks)
             K(c, TEA_K_EIG, 0.0, [&] { launch_eig_setup(kargs(c, b), s, c->stream); });
+        // the fused passes read the coefficients from constant memory (every block's copy
+        // is identical: they derive from globally reduced scalars)
+        if (use_tb(c, s)) CK(tb_coef_upload(c->coef_slot, c->blocks[0].S, c->stream));
         chain(c, s, true, false, F_R0, F_R0, false);
         read_state(c);
         if (!c->hS->done) {
@@ -1169,6 +1166,7 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
             ws += L.total;
         }
         CK(cudaStreamSynchronize(c->stream));
+        c->coef_slot = tb_slot_acquire();
         *out = c.release();
         return TEA_OK;
     } catch (const TeaError &e) {
@@ -1263,6 +1261,7 @@ tea_status tea_finalize(tea_ctx *ctx) {
     if (ctx->hS) cudaFreeHost(ctx->hS);
     if (ctx->comm) ncclCommDestroy(ctx->comm);
     if (ctx->stream) cudaStreamDestroy(ctx->stream);
+    tb_slot_release(ctx->coef_slot);
     delete ctx;
     return TEA_OK;
 }

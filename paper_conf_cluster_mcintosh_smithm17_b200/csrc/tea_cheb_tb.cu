@@ -23,7 +23,41 @@
 // Single-block only (no extended bounds); blocks with neighbours use the per-step kernels.
 #include "tea_internal.h"
 
+#include <mutex>
+
 namespace tea {
+
+// Chebyshev coefficients of the fused passes live in constant memory (one slot per
+// context): uniform per-step scalars then cost LDC through the constant cache instead
+// of shared-memory wavefronts on the L1TEX pipe the passes are bound by.
+// Uploaded once per solve after the eigen-estimate (tb_coef_upload).
+constexpr int kTbSlots = 16;
+__constant__ double c_tb_coef[kTbSlots][4][kMaxS];
+static_assert(offsetof(Scalars, cheb_cz) == offsetof(Scalars, cheb_cx) + kMaxS * sizeof(double) &&
+                  offsetof(Scalars, cheb_ca) == offsetof(Scalars, cheb_cx) + 3 * kMaxS * sizeof(double),
+              "folded coefficients must be contiguous [4][kMaxS]");
+static std::mutex g_slot_mu;
+static bool g_slot_used[kTbSlots];
+
+int tb_slot_acquire() {
+    std::lock_guard<std::mutex> g(g_slot_mu);
+    for (int i = 0; i < kTbSlots; ++i)
+        if (!g_slot_used[i]) {
+            g_slot_used[i] = true;
+            return i;
+        }
+    return -1;
+}
+void tb_slot_release(int slot) {
+    if (slot < 0 || slot >= kTbSlots) return;
+    std::lock_guard<std::mutex> g(g_slot_mu);
+    g_slot_used[slot] = false;
+}
+cudaError_t tb_coef_upload(int slot, const Scalars *S, cudaStream_t st) {
+    return cudaMemcpyToSymbolAsync(c_tb_coef, S->cheb_cx, sizeof(c_tb_coef[0]),
+                                   sizeof(c_tb_coef[0]) * (size_t)slot, cudaMemcpyDeviceToDevice,
+                                   st);
+}
 
 namespace {
 
@@ -143,7 +177,7 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
     double2(*ringKy)[kThreads] = ringKx + D;
     double2(*ringR)[kThreads] = ringKy + D;
     double2(*ringZ2)[kThreads] = ringR + D;
-    double(*coef)[M] = reinterpret_cast<double(*)[M]>(ringZ2 + 2);
+    const double(*coef)[kMaxS] = c_tb_coef[a.coef_slot];
 
     Scalars *S = a.S;
     if (S->done) {
@@ -164,13 +198,6 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
             }
             return;
         }
-    }
-    if (threadIdx.x < M) {
-        const int i = step0 - 1 + threadIdx.x;
-        coef[0][threadIdx.x] = S->cheb_cx[i];
-        coef[1][threadIdx.x] = S->cheb_cz[i];
-        coef[2][threadIdx.x] = S->cheb_cr[i];
-        coef[3][threadIdx.x] = S->cheb_ca[i];
     }
     const double2 z0 = make_double2(0.0, 0.0);
     for (int d = 0; d < D; ++d) {
@@ -292,19 +319,21 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
             // lane 0's left and lane 31's right neighbours are outside the strip: the
             // shuffles return the lane's own (finite) value, which only pollutes the
             // overlap columns every step already discards -- no selects needed
+            // x direction in flux form: A x = x + sum_faces K_f (x_c - x_f) (Listing 1
+            // regrouped). gw = Kx_w (x_A - x_left) is formed by the lane that owns the face's
+            // Kx; its east neighbour receives it as -(its east flux). Two shuffles of x and
+            // one of the flux -- no shuffle of Kx.
             const double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
-            const double right = __shfl_down_sync(0xffffffffu, xc.x, 1);
-            const double kxB = __shfl_down_sync(0xffffffffu, kx.x, 1);
+            const double gw = kx.x * (xc.x - left);
+            const double gm = kx.y * (xc.x - xc.y);
+            const double ge = __shfl_down_sync(0xffffffffu, gw, 1);  // Kx_e (x_right - x_B)
             // Dependency order: xp (the "up" row) is the row step t-1 produced in THIS
-            // row-iteration; everything else is older. Form the rest first, fold xp in
-            // last (A x = Listing 1; only the rounding order of the sums differs).
-            const double cx = coef[0][t - 1], cz = coef[1][t - 1], cr = coef[2][t - 1],
-                         ca = coef[3][t - 1];
+            // row-iteration; everything else is older. Form the rest first, fold xp in last.
+            const int ci = step0 - 2 + t;
+            const double cx = coef[0][ci], cz = coef[1][ci], cr = coef[2][ci], ca = coef[3][ci];
             double2 AXo, base;  // A x without the up term; the step's x-independent part
-            AXo.x = (1.0 + (kyn.x + kyc.x) + (kx.y + kx.x)) * xc.x - kyc.x * xm.x -
-                    (kx.y * xc.y + kx.x * left);
-            AXo.y = (1.0 + (kyn.y + kyc.y) + (kxB + kx.y)) * xc.y - kyc.y * xm.y -
-                    (kxB * right + kx.y * xc.x);
+            AXo.x = (1.0 + (kyn.x + kyc.x)) * xc.x - kyc.x * xm.x + (gw + gm);
+            AXo.y = (1.0 + (kyn.y + kyc.y)) * xc.y - kyc.y * xm.y - (gm + ge);
             base.x = cx * xc.x + cz * z2.x + cr * rq.x;
             base.y = cx * xc.y + cz * z2.y + cr * rq.y;
             double2 zn;
@@ -367,8 +396,7 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
     const int width = R.j1 - (R.j0 & ~1);
     const int nstrips = (width + G::OW - 1) / G::OW;
     dim3 grid((nstrips + kWarps - 1) / kWarps, (R.k1 - R.k0 + ty - 1) / ty);
-    constexpr size_t smem =
-        sizeof(double2) * (3 * G::D + 2) * kThreads + sizeof(double) * 4 * M;
+    constexpr size_t smem = sizeof(double2) * (3 * G::D + 2) * kThreads;
     static bool attr = false;  // per instantiation
     if (!attr) {
         cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST>,
@@ -401,6 +429,50 @@ static void tb_dispatch(const KArgs &a, const Region &R, const Region &Dd, int t
 }
 
 int tb_max_steps() { return 5; }
+
+// Rows per CTA tile: a CTA costs ~ (ty + 2M) row-iterations (pipeline fill/drain), all
+// CTAs are alike, so a launch costs ~ waves x (ty + 2M) with waves = ceil(ctas / slots).
+// Pick ty minimising that (slots = SMs x resident CTAs per SM of this kernel).
+int tb_auto_rows(int M, int width, int height) {
+    static int slots[8] = {};
+    M = M < 1 ? 1 : (M > kTbMaxSteps ? kTbMaxSteps : M);
+    if (!slots[M]) {
+        int dev = 0, nsm = 148, per = 0;
+        cudaGetDevice(&dev);
+        cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, dev);
+        const size_t smem = sizeof(double2) * (3 * 8 + 2) * kThreads;
+        cudaError_t e = cudaSuccess;
+        switch (M) {
+#define OCC(m)                                                                                   \
+    case m:                                                                                      \
+        cudaFuncSetAttribute(k_cheb_tb<m, false, false, true>,                                   \
+                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);            \
+        e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per, k_cheb_tb<m, false, false, true>, \
+                                                          kThreads, smem);                       \
+        break;
+            OCC(1) OCC(2) OCC(3) OCC(4) OCC(5)
+#undef OCC
+        }
+        if (e != cudaSuccess || per < 1) per = 1;
+        slots[M] = nsm * per;
+    }
+    const int ow = tb_out_cols(M);
+    const int gx = ((width + ow - 1) / ow + kWarps - 1) / kWarps;
+    int best = height, bestc = 0x7fffffff;
+    for (int w = 1; w <= 256; ++w) {
+        const int tiles = (int)((long long)slots[M] * w / gx);
+        if (tiles < 1) continue;
+        const int ty = (height + tiles - 1) / tiles;
+        const int waves = (int)(((long long)gx * ((height + ty - 1) / ty) + slots[M] - 1) / slots[M]);
+        const long long cost = (long long)waves * (ty + 2 * M);
+        if (cost < bestc) {
+            bestc = (int)cost;
+            best = ty;
+        }
+        if (ty <= 2 * M) break;
+    }
+    return best < 1 ? 1 : best;
+}
 
 int tb_ctas(int M, int width, int height, int ty) {
     const int ow = tb_out_cols(M);

@@ -82,6 +82,7 @@ struct KArgs {
     const double *kz;
     long long ps;
     int nz;
+    int coef_slot;  // constant-memory coefficient slot of the fused passes (tea_cheb_tb.cu)
 };
 
 Launch plan_stencil(const Region &R, int ty_req, int ncta_target);
@@ -158,6 +159,10 @@ void launch_cg1_w(const KArgs &a, const Launch &L, const Region &R, const double
 constexpr int kTbMaxSteps = 5;
 int tb_out_cols(int M);
 int tb_ctas(int M, int width, int height, int ty);
+int tb_auto_rows(int M, int width, int height);
+int tb_slot_acquire();  // -1: none free (the context then uses per-step kernels)
+void tb_slot_release(int slot);
+cudaError_t tb_coef_upload(int slot, const Scalars *S, cudaStream_t st);
 void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, int ty, int jlim,
                     int step0, bool first, bool fuse, bool last, bool restart, const double *rin,
                     const double *win, double *rout, const double *zin1, const double *zin2,
