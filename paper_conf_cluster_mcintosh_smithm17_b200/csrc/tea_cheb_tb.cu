@@ -146,6 +146,10 @@ __device__ bool grid_arrive2(unsigned *ticket) {
 constexpr int kTbUnroll = TEA_TB_UNROLL;  // measured: 2 (step t+1 of row k overlapping
                                           // step t of row k+1) costs registers, no gain
 
+// dynamic shared memory of a pass: the Kx, Ky, r delay rings (depth 8, one double2 per
+// thread and row)
+constexpr size_t tb_smem_bytes() { return sizeof(double2) * 3 * 8 * kThreads; }
+
 template <int M>
 struct TbGeom {
     static constexpr int MR = (M + 1) & ~1;  // margin, even (double2 alignment)
@@ -158,9 +162,16 @@ struct TbGeom {
 #define TEA_TB_MINB 1
 #endif
 #ifndef TEA_TB_REGLINES
-#define TEA_TB_REGLINES 0  // 1: register shift registers (measured slower: 225 regs,
-                            // 2 CTAs/SM, 737 vs 660 us/outer, profiles/r01_tb_reglines.txt)
+#define TEA_TB_REGLINES 0  // 1: Kx, Ky and r lines in registers (measured slower: 225 regs,
+                            // 2 CTAs/SM, 737 vs 660 us/outer, profiles/r01_tb_reglines.txt);
+                            // 2: r only
 #endif
+#define TB_REG_K (TEA_TB_REGLINES == 1)
+#ifndef TEA_TB_L2PF
+#define TEA_TB_L2PF 0  // rows of L2 bulk-prefetch distance (0 = off; 3, 6, 10 measured
+                       // slower: profiles/r01_tb_variants2.txt)
+#endif
+#define TB_REG_R (TEA_TB_REGLINES >= 1)
 template <int M, bool FIRST, bool FUSE, bool LAST>
 __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
     k_cheb_tb(const double *__restrict__ rin, const double *__restrict__ win,
@@ -176,7 +187,6 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
     double2(*ringKx)[kThreads] = reinterpret_cast<double2(*)[kThreads]>(tb_smem);
     double2(*ringKy)[kThreads] = ringKx + D;
     double2(*ringR)[kThreads] = ringKy + D;
-    double2(*ringZ2)[kThreads] = ringR + D;
     const double(*coef)[kMaxS] = c_tb_coef[a.coef_slot];
 
     Scalars *S = a.S;
@@ -205,11 +215,10 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
         ringKy[d][threadIdx.x] = z0;
         ringR[d][threadIdx.x] = z0;
     }
-    ringZ2[0][threadIdx.x] = z0;
-    ringZ2[1][threadIdx.x] = z0;
     __syncthreads();
 
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5, tid = threadIdx.x;
+    (void)tid;
     const int strip = blockIdx.x * kWarps + warp;
     // strips tile the output region R (which may reach into the halo on sides with a
     // neighbour block: extended bounds); first strip starts MR before it
@@ -249,16 +258,48 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
         pKy = ldg2c(Ky + o);
     };
     if (kt0 < kt1) load(orow);
+#if TEA_TB_L2PF
+    // L2 prefetch TEA_TB_L2PF rows ahead through the TMA unit (one lane, no registers, no
+    // L1TEX wavefronts): the one-row register prefetch then hits L2
+    const int jA0 = __shfl_sync(0xffffffffu, jA, 0);
+    int pfb = (jlim - jA0) * 8;
+    pfb = pfb > kStrip * 8 ? kStrip * 8 : (pfb & ~15);
+    auto l2pf = [&](const double *base, long long o) {
+        asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(base + o), "r"(pfb)
+                     : "memory");
+    };
+#endif
     int head = 0;  // ring slot of row k
-#if TEA_TB_REGLINES
-    double2 rKx[M + 1], rKy[M + 1], rR[M + 1], z2prev = z0;
+    double2 z2prev = z0;  // z_{i-2} input of the previous row (a one-row register delay)
+#if TB_REG_K
+    double2 rKx[M + 1], rKy[M + 1];
 #pragma unroll
-    for (int i = 0; i <= M; ++i) rKx[i] = rKy[i] = rR[i] = z0;
+    for (int i = 0; i <= M; ++i) rKx[i] = rKy[i] = z0;
+#endif
+#if TB_REG_R
+    double2 rR[M + 1];
+#pragma unroll
+    for (int i = 0; i <= M; ++i) rR[i] = z0;
 #endif
 #pragma unroll(kTbUnroll)
     for (int k = kbeg; k < kend; ++k, orow += pitch, head = (head + 1) & (D - 1)) {
         double2 X = pX, Wv = pW, Z2 = pZ2, KX = pKx, KY = pKy, RR = pR;
         if (k + 1 < kend) load(orow + pitch);
+#if TEA_TB_L2PF
+        if (lane == 0 && pfb > 0 && k + TEA_TB_L2PF < kend) {
+            const long long o = orow + (long long)TEA_TB_L2PF * pitch;
+            if (FIRST) {
+                l2pf(rin, o);
+                if (FUSE) l2pf(win, o);
+            } else {
+                l2pf(zin1, o);
+                l2pf(zin2, o);
+                l2pf(rin, o);
+            }
+            l2pf(Kx, o);
+            l2pf(Ky, o);
+        }
+#endif
         double2 rk;
         if (FIRST) {
             if (FUSE) X = make_double2(X.x - alpha * Wv.x, X.y - alpha * Wv.y);
@@ -267,54 +308,56 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
         } else {
             rk = RR;
         }
-#if TEA_TB_REGLINES
-        // delay lines as register shift registers: index i holds row k - i (the step
-        // loop is unrolled, so step t's lag t is a compile-time index) -- register moves
-        // on the ALU pipes instead of shared-memory wavefronts through L1TEX
+        // delay lines: shared-memory rings, or register shift registers (index i holds
+        // row k - i; the step loop is unrolled, so step t's lag t is a compile-time index)
+#if TB_REG_K
 #pragma unroll
         for (int i = M; i > 0; --i) {
             rKx[i] = rKx[i - 1];
             rKy[i] = rKy[i - 1];
-            rR[i] = rR[i - 1];
         }
         rKx[0] = KX;
         rKy[0] = KY;
-        rR[0] = rk;
-        const double2 z2row = z2prev;  // z_{i-2} of row k-1
-        if (!FIRST) z2prev = Z2;
 #else
         ringKx[head][tid] = KX;
         ringKy[head][tid] = KY;
-        ringR[head][tid] = rk;
-        if (!FIRST) ringZ2[k & 1][tid] = Z2;
 #endif
+#if TB_REG_R
+#pragma unroll
+        for (int i = M; i > 0; --i) rR[i] = rR[i - 1];
+        rR[0] = rk;
+#else
+        ringR[head][tid] = rk;
+#endif
+        const double2 z2row = z2prev;  // z_{i-2} of row k-1
+        if (!FIRST) z2prev = Z2;
         W[0][0] = W[0][1];
         W[0][1] = W[0][2];
         W[0][2] = X;
 #pragma unroll
         for (int t = 1; t <= M; ++t) {
             const int q = k - t;
-#if TEA_TB_REGLINES
-            const double2 kx = rKx[t], kyc = rKy[t], kyn = rKy[t - 1], rq = rR[t];
+            const int sq = (head - t) & (D - 1), sq1 = (head - t + 1) & (D - 1);
+#if TB_REG_K
+            const double2 kx = rKx[t], kyc = rKy[t], kyn = rKy[t - 1];
+#else
+            const double2 kx = ringKx[sq][tid];
+            const double2 kyc = ringKy[sq][tid];
+            const double2 kyn = ringKy[sq1][tid];
+#endif
+#if TB_REG_R
+            const double2 rq = rR[t];
+#else
+            const double2 rq = ringR[sq][tid];
+#endif
+            (void)sq;
+            (void)sq1;
             double2 z2;
             if (t == 1) {
                 z2 = FIRST ? z0 : z2row;
             } else {
                 z2 = W[t >= 2 ? t - 2 : 0][0];
             }
-#else
-            const int sq = (head - t) & (D - 1), sq1 = (head - t + 1) & (D - 1);
-            const double2 kx = ringKx[sq][tid];
-            const double2 kyc = ringKy[sq][tid];
-            const double2 kyn = ringKy[sq1][tid];
-            const double2 rq = ringR[sq][tid];
-            double2 z2;
-            if (t == 1) {
-                z2 = FIRST ? z0 : ringZ2[(k + 1) & 1][tid];  // row k-1
-            } else {
-                z2 = W[t >= 2 ? t - 2 : 0][0];
-            }
-#endif
             const double2 xm = W[t - 1][0], xc = W[t - 1][1], xp = W[t - 1][2];
             // lane 0's left and lane 31's right neighbours are outside the strip: the
             // shuffles return the lane's own (finite) value, which only pollutes the
@@ -396,7 +439,7 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
     const int width = R.j1 - (R.j0 & ~1);
     const int nstrips = (width + G::OW - 1) / G::OW;
     dim3 grid((nstrips + kWarps - 1) / kWarps, (R.k1 - R.k0 + ty - 1) / ty);
-    constexpr size_t smem = sizeof(double2) * (3 * G::D + 2) * kThreads;
+    constexpr size_t smem = tb_smem_bytes();
     static bool attr = false;  // per instantiation
     if (!attr) {
         cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST>,
@@ -440,7 +483,7 @@ int tb_auto_rows(int M, int width, int height) {
         int dev = 0, nsm = 148, per = 0;
         cudaGetDevice(&dev);
         cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, dev);
-        const size_t smem = sizeof(double2) * (3 * 8 + 2) * kThreads;
+        const size_t smem = tb_smem_bytes();
         cudaError_t e = cudaSuccess;
         switch (M) {
 #define OCC(m)                                                                                   \
