@@ -537,15 +537,6 @@ int tb_steps(const tea_ctx *c) {
     return std::min(m, kTbMaxSteps);
 }
 
-// u += alpha p in the first fused pass instead of the SpMV (TEA_UMOVE=1; measurement knob)
-bool tb_umove() {
-    static bool v = [] {
-        const char *e = getenv("TEA_UMOVE");
-        return e ? atoi(e) != 0 : false;
-    }();
-    return v;
-}
-
 bool single_block(tea_ctx *c) { return c->px * c->py == 1; }
 bool is3d(const tea_ctx *c) { return c->blocks[0].L.nz > 1; }
 
@@ -556,9 +547,8 @@ bool is3d(const tea_ctx *c) { return c->blocks[0].L.nz > 1; }
 // depth d >= s + 1 (corners included); pass p then runs on bounds extended by
 // 1 + (steps after it), so the last pass leaves z_s valid on the 1-cell ring the next
 // SpMV reads; no z exchange. (One block: every extension is empty.)
-// fused: the first pass also does r_out = r_in - alpha w and u += alpha p (p in field pnew).
 int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout,
-                  bool sets_cond, int pnew) {
+                  bool sets_cond) {
     const auto passes = tb_passes(s, tb_steps(c));
     const int pairA[2] = {F_Z0, F_Z2}, pairB[2] = {F_Z1, F_Z3};
     const bool blocks = !single_block(c);
@@ -578,17 +568,15 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
             int ty = c->opts.tb_rows > 0 ? c->opts.tb_rows : 0;
             // tall tiles keep the 2M-row pipeline fill small; whole waves (tb_auto_rows)
             if (ty <= 0) ty = tb_auto_rows(M, R.j1 - R.j0, R.k1 - R.k0);
-            const bool um = fu && pnew >= 0;
-            int streams = first ? (fu ? (um ? 6 : 4) : 3) : 5;  // reads (um: r, w, p, u, Kx, Ky)
-            streams += (fu ? 1 : 0) + (um ? 1 : 0) + (last ? 1 : 2);  // r', u, z_last(, z_{last-1})
+            int streams = first ? (fu ? 4 : 3) : 5;     // reads
+            streams += (fu ? 1 : 0) + (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})
             const int kid = last ? TEA_K_TB_LAST : (first ? TEA_K_TB_FIRST : TEA_K_TB_MID);
             K(c, kid, sbytes(b, streams), [&] {
                 launch_cheb_tb(kargs(c, b, last && sets_cond), R, D, M, ty, jlim, step0, first,
                                fu, last, restart, b.f[first && fu ? rin : r], b.f[F_W],
                                b.f[rout], first ? nullptr : b.f[pairB[in]],
                                first ? nullptr : b.f[pairA[in]], b.f[pairA[o]], b.f[pairB[o]],
-                               b.f[F_KX], b.f[F_KY], um ? b.f[pnew] : nullptr,
-                               um ? b.f[F_U] : nullptr, c->stream);
+                               b.f[F_KX], b.f[F_KY], c->stream);
             });
         }
         step0 += M;
@@ -605,9 +593,8 @@ bool use_tb(tea_ctx *c, int s) {
     return single_block(c) || c->d >= s + 1;
 }
 
-int chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond,
-          int pnew = -1) {
-    if (use_tb(c, s)) return cheb_chain_tb(c, s, restart, fused, rin, rout, sets_cond, pnew);
+int chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond) {
+    if (use_tb(c, s)) return cheb_chain_tb(c, s, restart, fused, rin, rout, sets_cond);
     return cheb_chain(c, s, restart, fused, rin, rout, sets_cond);
 }
 
@@ -622,21 +609,18 @@ int zs_field(tea_ctx *c, int s) {
 
 void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
     const bool fused = single_block(c);
-    // fused passes: u += alpha p moves from the SpMV (HBM-bound) into the first pass
-    // (L1TEX-bound, HBM headroom): SpMV 8 -> 6 streams, first pass 7 -> 10
-    const bool umove = fused && use_tb(c, s) && tb_umove();
     const int zs = zs_field(c, s);
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan_st(c, b, R);
-        K(c, TEA_K_SPMV, sbytes(b, umove ? 6 : 8), [&] {
+        K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[zs], b.f[F_P0 + par], b.f[F_P1 - par],
-                        b.f[F_W], umove ? nullptr : b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
+                        b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
         });
     }
     reduce(c, 0, 1);
     if (fused) {
-        chain(c, s, false, true, F_R0 + par, F_R1 - par, sets_cond, umove ? F_P1 - par : -1);
+        chain(c, s, false, true, F_R0 + par, F_R1 - par, sets_cond);
     } else {
         for (auto &b : c->blocks) {
             Region R = b.owned();

@@ -24,8 +24,6 @@
 #include "tea_internal.h"
 
 #include <mutex>
-#include <type_traits>
-#include <cstdlib>
 
 namespace tea {
 
@@ -145,7 +143,6 @@ __device__ bool grid_arrive2(unsigned *ticket) {
 #ifndef TEA_TB_UNROLL
 #define TEA_TB_UNROLL 1
 #endif
-__host__ __device__ constexpr int md(int x, int m) { return ((x % m) + m) % m; }
 constexpr int kTbUnroll = TEA_TB_UNROLL;  // measured: 2 (step t+1 of row k overlapping
                                           // step t of row k+1) costs registers, no gain
 
@@ -181,8 +178,7 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
               double *__restrict__ rout, const double *__restrict__ zin1,
               const double *__restrict__ zin2, double *__restrict__ zoutA,
               double *__restrict__ zoutB, const double *__restrict__ Kx,
-              const double *__restrict__ Ky, const double *__restrict__ pin,
-              double *__restrict__ u, KArgs a, Region R, Region Dd, int ty, int jlim,
+              const double *__restrict__ Ky, KArgs a, Region R, Region Dd, int ty, int jlim,
               int step0, int restart) {
     using G = TbGeom<M>;
     constexpr int D = G::D;
@@ -246,8 +242,6 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
 
     // prefetch registers for input row k; running element offsets (no k*pitch products)
     double2 pX = z0, pW = z0, pZ2 = z0, pKx = z0, pKy = z0, pR = z0;
-    (void)pin;
-    (void)u;  // the u update rides on k_cheb_tma<..., UMOVE> only
     const int kbeg = kt0 - M, kend = kt1 + M;
     long long orow = (long long)kbeg * pitch + jA;  // offset of (jA, k)
     auto load = [&](long long o) {
@@ -430,529 +424,9 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
     }
 }
 
-// ------------------------------------------------------------------ phase-unrolled passes
-// k_cheb_tb with the row loop unrolled by P = 6 (>= M + 1 rows of delay, a multiple of the
-// 3-row stencil window): ring slots and window rows become compile-time indices, so the
-// per-row window shifts (register moves) and ring-slot arithmetic of k_cheb_tb disappear
-// (SASS: 316 -> see DESIGN.md §4.4 instructions per row-iteration). Same loads, same
-// shared-memory delay lines (depth 6), same arithmetic and results bit for bit.
-#ifndef TEA_TB6_MINB
-#define TEA_TB6_MINB 1
-#endif
-#ifndef TEA_TB6_REGR
-#define TEA_TB6_REGR 0  // r delay line in registers instead of shared memory
-#endif
-#ifndef TEA_TB6_REGKX
-#define TEA_TB6_REGKX 0  // Kx delay line in registers
-#endif
-constexpr size_t tb6_smem_bytes() { return sizeof(double2) * 3 * 6 * kThreads; }
-
-template <int M, bool FIRST, bool FUSE, bool LAST>
-__global__ void __launch_bounds__(kThreads, TEA_TB6_MINB)
-    k_cheb_tb6(const double *__restrict__ rin, const double *__restrict__ win,
-               double *__restrict__ rout, const double *__restrict__ zin1,
-               const double *__restrict__ zin2, double *__restrict__ zoutA,
-               double *__restrict__ zoutB, const double *__restrict__ Kx,
-               const double *__restrict__ Ky, KArgs a, Region R, Region Dd, int ty, int jlim,
-               int step0, int restart) {
-    using G = TbGeom<M>;
-    constexpr int P = 6;
-    static_assert(M <= 5, "delay of M + 1 rows fits the period");
-    extern __shared__ double2 tb_smem[];
-    double2(*ringKx)[kThreads] = reinterpret_cast<double2(*)[kThreads]>(tb_smem);
-    double2(*ringKy)[kThreads] = ringKx + P;
-    double2(*ringR)[kThreads] = ringKy + P;
-    const double(*coef)[kMaxS] = c_tb_coef[a.coef_slot];
-
-    Scalars *S = a.S;
-    if (S->done) {
-        if (LAST && blockIdx.x == 0 && blockIdx.y == 0 && threadIdx.x == 0 && a.set_cond && a.cond)
-            cudaGraphSetConditional(a.cond, 0u);
-        return;
-    }
-    double alpha = 0.0;
-    if (FUSE) {
-        const double pw = S->red_pw;
-        alpha = S->gam_old / pw;
-        if (!(pw > 0.0) || !isfinite(alpha)) {
-            if (grid_arrive2(&S->ticket) && threadIdx.x == 0) {
-                S->done = 1;
-                S->status = DS_BREAKDOWN;
-                if (LAST && a.set_cond && a.cond) cudaGraphSetConditional(a.cond, 0u);
-            }
-            return;
-        }
-    }
-    const double2 z0 = make_double2(0.0, 0.0);
-    const int tid = threadIdx.x;
-#pragma unroll
-    for (int d = 0; d < P; ++d) {
-        ringKx[d][tid] = z0;
-        ringKy[d][tid] = z0;
-        ringR[d][tid] = z0;
-    }
-    // each thread reads back only its own slots: no barrier needed
-    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    const int strip = blockIdx.x * kWarps + warp;
-    const int jA = (R.j0 & ~1) - G::MR + strip * G::OW + 2 * lane;
-    const int kt0 = R.k0 + blockIdx.y * ty;
-    const int kt1 = min(kt0 + ty, R.k1);
-    const int pitch = a.pitch;
-    const bool ld_ok = jA + 1 < jlim;
-    const int cA = 2 * lane, cB = 2 * lane + 1;
-    const bool oA = cA >= G::MR && cA < kStrip - G::MR && jA >= R.j0 && jA < R.j1;
-    const bool oB = cB >= G::MR && cB < kStrip - G::MR && jA + 1 >= R.j0 && jA + 1 < R.j1;
-    const bool dA = oA && jA >= Dd.j0 && jA < Dd.j1, dB = oB && jA + 1 >= Dd.j0 && jA + 1 < Dd.j1;
-
-    double2 W[M][3];
-#pragma unroll
-    for (int t = 0; t < M; ++t) W[t][0] = W[t][1] = W[t][2] = z0;
-    double2 Z2r[2] = {z0, z0};
-#if TEA_TB6_REGKX
-    double2 lineKx[P];
-#pragma unroll
-    for (int i = 0; i < P; ++i) lineKx[i] = z0;
-#endif
-#if TEA_TB6_REGR
-    double2 lineR[P];
-#pragma unroll
-    for (int i = 0; i < P; ++i) lineR[i] = z0;
-#endif
-    double dot0 = 0.0, dot1 = 0.0;
-
-    // prefetch registers, double-buffered by phase parity (no copies): X, W or z_{i-2},
-    // Kx, Ky, r
-    double2 pf[2][5];
-#pragma unroll
-    for (int i = 0; i < 5; ++i) pf[0][i] = pf[1][i] = z0;
-    const int kbeg = kt0 - M, kend = kt1 + M;
-    const int nrows = kt0 < kt1 ? kend - kbeg : 0;
-    long long orow = (long long)kbeg * pitch + jA;
-    // rows up to kend are inside the allocation (H >= M + 2), so the one-row-ahead load
-    // of the last iteration needs no guard
-    auto load = [&](double2 *f, long long o) {
-        if (!ld_ok) return;
-        if (FIRST) {
-            f[0] = ldg2c(rin + o);
-            if (FUSE) f[1] = ldg2c(win + o);
-        } else {
-            f[0] = ldg2c(zin1 + o);
-            f[4] = ldg2c(rin + o);
-        }
-        f[2] = ldg2c(Kx + o);
-        f[3] = ldg2c(Ky + o);
-    };
-    if (nrows > 0) load(pf[0], orow);
-
-    auto body = [&](auto phc, int ki) {
-        constexpr int ph = decltype(phc)::value;
-        const int k = kbeg + ki;
-        double2 *cur = pf[ph % 2];
-        double2 X = cur[0];
-        const double2 Wv = cur[1], KX = cur[2], KY = cur[3], RR = cur[4];
-        load(pf[(ph + 1) % 2], orow + pitch);
-        double2 rk;
-        if (FIRST) {
-            if (FUSE) X = make_double2(X.x - alpha * Wv.x, X.y - alpha * Wv.y);
-            rk = X;
-            if (FUSE && k >= kt0 && k < kt1) st2m(rout + orow, X, oA, oB);
-        } else {
-            rk = RR;
-            // z_{i-2} of row k is first needed one row-iteration later (step 1 of row k):
-            // loaded here, un-prefetched, into the slot read at the next phase
-            if (ld_ok) Z2r[ph % 2] = ldg2c(zin2 + orow);
-        }
-#if TEA_TB6_REGKX
-        lineKx[ph] = KX;
-#else
-        ringKx[ph][tid] = KX;
-#endif
-        ringKy[ph][tid] = KY;
-#if TEA_TB6_REGR
-        lineR[ph] = rk;
-#else
-        ringR[ph][tid] = rk;
-#endif
-        W[0][ph % 3] = X;
-#pragma unroll
-        for (int t = 1; t <= M; ++t) {
-            const int q = k - t;
-#if TEA_TB6_REGKX
-            const double2 kx = lineKx[md(ph - t, P)];
-#else
-            const double2 kx = ringKx[md(ph - t, P)][tid];
-#endif
-            const double2 kyc = ringKy[md(ph - t, P)][tid];
-            const double2 kyn = ringKy[md(ph - t + 1, P)][tid];
-#if TEA_TB6_REGR
-            const double2 rq = lineR[md(ph - t, P)];
-#else
-            const double2 rq = ringR[md(ph - t, P)][tid];
-#endif
-            double2 z2;
-            if (t == 1)
-                z2 = FIRST ? z0 : Z2r[(ph + 1) % 2];
-            else
-                z2 = W[t >= 2 ? t - 2 : 0][md(ph - t, 3)];
-            const double2 xm = W[t - 1][md(ph - t - 1, 3)];
-            const double2 xc = W[t - 1][md(ph - t, 3)];
-            const double2 xp = W[t - 1][md(ph - t + 1, 3)];
-            const double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
-            const double gw = kx.x * (xc.x - left);
-            const double gm = kx.y * (xc.x - xc.y);
-            const double ge = __shfl_down_sync(0xffffffffu, gw, 1);
-            const int ci = step0 - 2 + t;
-            const double cx = coef[0][ci], cz = coef[1][ci], cr = coef[2][ci], ca = coef[3][ci];
-            double2 AXo, base;
-            AXo.x = (1.0 + (kyn.x + kyc.x)) * xc.x - kyc.x * xm.x + (gw + gm);
-            AXo.y = (1.0 + (kyn.y + kyc.y)) * xc.y - kyc.y * xm.y - (gm + ge);
-            base.x = cx * xc.x + cz * z2.x + cr * rq.x;
-            base.y = cx * xc.y + cz * z2.y + cr * rq.y;
-            double2 zn;
-            zn.x = fma(-ca, fma(-kyn.x, xp.x, AXo.x), base.x);
-            zn.y = fma(-ca, fma(-kyn.y, xp.y, AXo.y), base.y);
-            const bool rowout = q >= kt0 && q < kt1;
-            if (t < M) {
-                W[t < M ? t : 0][md(ph - t, 3)] = zn;
-                if (t == M - 1 && !LAST && rowout) st2m(zoutA + (orow - t * pitch), zn, oA, oB);
-            } else if (rowout) {
-                st2m(zoutB + (orow - t * pitch), zn, oA, oB);
-                if (LAST && q >= Dd.k0 && q < Dd.k1) {
-                    if (dA) {
-                        dot0 += rq.x * zn.x;
-                        dot1 += rq.x * rq.x;
-                    }
-                    if (dB) {
-                        dot0 += rq.y * zn.y;
-                        dot1 += rq.y * rq.y;
-                    }
-                }
-            }
-        }
-        orow += pitch;
-    };
-    for (int kk = 0; kk < nrows; kk += P) {
-        body(std::integral_constant<int, 0>{}, kk);
-        if (kk + 1 < nrows) body(std::integral_constant<int, 1>{}, kk + 1);
-        if (kk + 2 < nrows) body(std::integral_constant<int, 2>{}, kk + 2);
-        if (kk + 3 < nrows) body(std::integral_constant<int, 3>{}, kk + 3);
-        if (kk + 4 < nrows) body(std::integral_constant<int, 4>{}, kk + 4);
-        if (kk + 5 < nrows) body(std::integral_constant<int, 5>{}, kk + 5);
-    }
-    if (LAST) {
-        double t0, t1;
-        if (grid_reduce2(dot0, dot1, a.partials, &S->ticket, &t0, &t1)) {
-            if (threadIdx.x == 0) {
-                S->red_gam = t0;
-                S->red_rr = t1;
-                if (FUSE) S->alpha_prev = alpha;
-                if (!restart) {
-                    S->it += 1;
-                    S->outer += 1;
-                }
-            }
-        }
-    } else if (FUSE) {
-        if (blockIdx.x == 0 && blockIdx.y == 0 && threadIdx.x == 0) S->alpha_prev = alpha;
-    }
-}
-
-// ------------------------------------------------------------------ TMA-fed passes
-// Same schedule and arithmetic as k_cheb_tb, different data movement:
-// * every input row of a warp's strip arrives by TMA bulk copies (cp.async.bulk, one
-//   per stream and row, issued by lane 0) into a per-warp NS-stage shared-memory ring
-//   guarded by mbarriers (expect_tx) -- NS-1 rows in flight per warp, no load registers,
-//   no LSU wavefronts for the global reads, no shared-memory stores;
-// * each lane moves its double2 of the row into registers once; the delay lines
-//   (Kx, Ky, r, z_{i-2}) and the stencil windows are REGISTER arrays rotated by
-//   compile-time indices: the row loop is unrolled by P = 6 (>= M+1, a multiple of 3),
-//   so no shift moves and no shared-memory delay-line traffic.
-namespace {
-__device__ __forceinline__ unsigned smem_u32(const void *p) {
-    return static_cast<unsigned>(__cvta_generic_to_shared(p));
-}
-__device__ __forceinline__ void mbar_init(unsigned bar, unsigned count) {
-    asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(bar), "r"(count) : "memory");
-}
-__device__ __forceinline__ void mbar_expect_tx(unsigned bar, unsigned bytes) {
-    asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(bar), "r"(bytes)
-                 : "memory");
-}
-__device__ __forceinline__ void mbar_wait(unsigned bar, unsigned parity) {
-    asm volatile(
-        "{\n\t.reg .pred p;\n"
-        "TEA_MBW_%=:\n\t"
-        "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n\t"
-        "@!p bra TEA_MBW_%=;\n}\n" ::"r"(bar),
-        "r"(parity)
-        : "memory");
-}
-__device__ __forceinline__ void bulk_g2s(unsigned dst, const void *src, unsigned bytes,
-                                         unsigned bar) {
-    asm volatile(
-        "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
-            dst),
-        "l"(src), "r"(bytes), "r"(bar)
-        : "memory");
-}
-__device__ __forceinline__ void fence_proxy_async() {
-    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
-}
-}  // namespace
-
-#ifndef TEA_TMA_STAGES
-#define TEA_TMA_STAGES 4
-#endif
-#ifndef TEA_TMA_MINB
-#define TEA_TMA_MINB 1
-#endif
-constexpr int kTmaStages = TEA_TMA_STAGES;
-
-// streams per row: FIRST: X = r, [w], Kx, Ky, [p, u]; otherwise X = z_{i-1}, z_{i-2}, r, Kx, Ky
-template <bool FIRST, bool FUSE, bool UMOVE>
-struct TmaStreams {
-    static constexpr int N = FIRST ? (FUSE ? (UMOVE ? 6 : 4) : 3) : 5;
-    static constexpr int KX = FIRST ? (FUSE ? 2 : 1) : 3;
-    static constexpr int KY = KX + 1;
-};
-template <bool FIRST, bool FUSE, bool UMOVE>
-constexpr size_t tma_smem_bytes() {
-    return (size_t)kWarps * kTmaStages * (TmaStreams<FIRST, FUSE, UMOVE>::N * 512 + 8);
-}
-
-template <int M, bool FIRST, bool FUSE, bool LAST, bool UMOVE>
-__global__ void __launch_bounds__(kThreads, TEA_TMA_MINB)
-    k_cheb_tma(const double *__restrict__ rin, const double *__restrict__ win,
-               double *__restrict__ rout, const double *__restrict__ zin1,
-               const double *__restrict__ zin2, double *__restrict__ zoutA,
-               double *__restrict__ zoutB, const double *__restrict__ Kx,
-               const double *__restrict__ Ky, const double *__restrict__ pin,
-               double *__restrict__ u, KArgs a, Region R, Region Dd, int ty, int jlim, int step0,
-               int restart) {
-    using G = TbGeom<M>;
-    using SS = TmaStreams<FIRST, FUSE, UMOVE>;
-    constexpr int NS = kTmaStages, NSTR = SS::N;
-    constexpr int P = 6;  // register rotation period (>= M + 1, multiple of 3)
-    static_assert(M <= 5, "rotation period 6 holds M + 1 rows");
-    static_assert(!UMOVE || (FIRST && FUSE), "u update rides on the fused first pass");
-    extern __shared__ __align__(16) unsigned char tma_smem[];
-    const double(*coef)[kMaxS] = c_tb_coef[a.coef_slot];
-
-    Scalars *S = a.S;
-    if (S->done) {
-        if (LAST && blockIdx.x == 0 && blockIdx.y == 0 && threadIdx.x == 0 && a.set_cond && a.cond)
-            cudaGraphSetConditional(a.cond, 0u);
-        return;
-    }
-    double alpha = 0.0;
-    if (FUSE) {
-        const double pw = S->red_pw;
-        alpha = S->gam_old / pw;
-        if (!(pw > 0.0) || !isfinite(alpha)) {
-            if (grid_arrive2(&S->ticket) && threadIdx.x == 0) {
-                S->done = 1;
-                S->status = DS_BREAKDOWN;
-                if (LAST && a.set_cond && a.cond) cudaGraphSetConditional(a.cond, 0u);
-            }
-            return;
-        }
-    }
-    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    double2 *stg = reinterpret_cast<double2 *>(tma_smem) + (size_t)warp * NS * NSTR * 32;
-    uint64_t *bars = reinterpret_cast<uint64_t *>(tma_smem + (size_t)kWarps * NS * NSTR * 512) +
-                     warp * NS;
-    const double2 z0 = make_double2(0.0, 0.0);
-
-    const int strip = blockIdx.x * kWarps + warp;
-    const int jA0 = (R.j0 & ~1) - G::MR + strip * G::OW;  // lane 0's first column
-    const int jA = jA0 + 2 * lane;
-    const int kt0 = R.k0 + blockIdx.y * ty;
-    const int kt1 = min(kt0 + ty, R.k1);
-    const int pitch = a.pitch;
-    const int cA = 2 * lane, cB = 2 * lane + 1;
-    const bool oA = cA >= G::MR && cA < kStrip - G::MR && jA >= R.j0 && jA < R.j1;
-    const bool oB = cB >= G::MR && cB < kStrip - G::MR && jA + 1 >= R.j0 && jA + 1 < R.j1;
-    const bool dA = oA && jA >= Dd.j0 && jA < Dd.j1, dB = oB && jA + 1 >= Dd.j0 && jA + 1 < Dd.j1;
-    // bytes of a row segment inside the allocation (16-B granules; lanes past it read 0)
-    int nb = (jlim - jA0) * 8;
-    nb = nb > kStrip * 8 ? kStrip * 8 : (nb < 0 ? 0 : (nb & ~15));
-    const int kbeg = kt0 - M, kend = kt1 + M;
-    const int nrows = kt0 < kt1 ? kend - kbeg : 0;
-    const bool wload = nb > 0 && nrows > 0;
-
-    // ring init: zero this lane's slots, barriers, then order both before the async proxy
-#pragma unroll
-    for (int i = 0; i < NS * NSTR; ++i) stg[i * 32 + lane] = z0;
-    if (lane == 0)
-        for (int s = 0; s < NS; ++s) mbar_init(smem_u32(&bars[s]), 1u);
-    __syncwarp();
-    if (lane == 0) fence_proxy_async();
-    __syncwarp();
-
-    const double *src[NSTR];
-    if (FIRST) {
-        src[0] = rin;
-        if constexpr (FUSE) src[1] = win;
-        if constexpr (UMOVE) {
-            src[4] = pin;
-            src[5] = u;
-        }
-    } else {
-        src[0] = zin1;
-        if constexpr (!FIRST) {
-            src[1] = zin2;
-            src[2] = rin;
-        }
-    }
-    src[SS::KX] = Kx;
-    src[SS::KY] = Ky;
-    auto issue = [&](int ki, int s) {
-        const unsigned bar = smem_u32(&bars[s]);
-        mbar_expect_tx(bar, (unsigned)(NSTR * nb));
-        const long long o = (long long)(kbeg + ki) * pitch + jA0;
-        const unsigned dst = smem_u32(stg + (size_t)s * NSTR * 32);
-#pragma unroll
-        for (int i = 0; i < NSTR; ++i) bulk_g2s(dst + i * 512, src[i] + o, (unsigned)nb, bar);
-    };
-    if (wload && lane == 0)
-        for (int i = 0; i < NS && i < nrows; ++i) issue(i, i);
-
-    // register state: stencil windows W[t][row % 3] (W[0] = input operand), delay lines
-    // indexed by row % P
-    double2 W[M][3];
-    double2 KXr[P], KYr[P], RRr[P], Z2r[2];
-#pragma unroll
-    for (int t = 0; t < M; ++t) W[t][0] = W[t][1] = W[t][2] = z0;
-#pragma unroll
-    for (int i = 0; i < P; ++i) KXr[i] = KYr[i] = RRr[i] = z0;
-    Z2r[0] = Z2r[1] = z0;
-    double dot0 = 0.0, dot1 = 0.0;
-
-    auto body = [&](auto phc, int ki) {
-        constexpr int ph = decltype(phc)::value;
-        const int k = kbeg + ki;
-        const long long orow = (long long)k * pitch + jA;
-        const int s = ki % NS;
-        if (wload) mbar_wait(smem_u32(&bars[s]), (unsigned)((ki / NS) & 1));
-        const double2 *row = stg + (size_t)s * NSTR * 32 + lane;
-        double2 X = row[0];
-        KXr[ph] = row[SS::KX * 32];
-        KYr[ph] = row[SS::KY * 32];
-        if (FIRST) {
-            if (FUSE) {
-                const double2 Wv = row[32];
-                X = make_double2(X.x - alpha * Wv.x, X.y - alpha * Wv.y);
-            }
-            RRr[ph] = X;
-            if (FUSE && k >= kt0 && k < kt1) {
-                st2m(rout + orow, X, oA, oB);
-                if (UMOVE && k >= Dd.k0 && k < Dd.k1) {
-                    const double2 Pv = row[4 * 32], Uv = row[5 * 32];
-                    st2m(u + orow, make_double2(Uv.x + alpha * Pv.x, Uv.y + alpha * Pv.y), dA,
-                         dB);
-                }
-            }
-        } else {
-            Z2r[ph % 2] = row[32];
-            RRr[ph] = row[64];
-        }
-        // the stage of the previous row is free (its values are in registers): refill
-        // it with the row NS - 1 ahead of this one
-        if (wload) {
-            __syncwarp();
-            if (lane == 0 && ki >= 1 && ki - 1 + NS < nrows) {
-                fence_proxy_async();
-                issue(ki - 1 + NS, (ki - 1) % NS);
-            }
-        }
-        W[0][ph % 3] = X;
-#pragma unroll
-        for (int t = 1; t <= M; ++t) {
-            const int q = k - t;
-            const double2 kx = KXr[md(ph - t, P)];
-            const double2 kyc = KYr[md(ph - t, P)];
-            const double2 kyn = KYr[md(ph - t + 1, P)];
-            const double2 rq = RRr[md(ph - t, P)];
-            double2 z2;
-            if (t == 1)
-                z2 = FIRST ? z0 : Z2r[(ph + 1) % 2];
-            else
-                z2 = W[t >= 2 ? t - 2 : 0][md(ph - t, 3)];
-            const double2 xm = W[t - 1][md(ph - t - 1, 3)];
-            const double2 xc = W[t - 1][md(ph - t, 3)];
-            const double2 xp = W[t - 1][md(ph - t + 1, 3)];
-            const double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
-            const double gw = kx.x * (xc.x - left);
-            const double gm = kx.y * (xc.x - xc.y);
-            const double ge = __shfl_down_sync(0xffffffffu, gw, 1);
-            const int ci = step0 - 2 + t;
-            const double cx = coef[0][ci], cz = coef[1][ci], cr = coef[2][ci], ca = coef[3][ci];
-            double2 AXo, base;
-            AXo.x = (1.0 + (kyn.x + kyc.x)) * xc.x - kyc.x * xm.x + (gw + gm);
-            AXo.y = (1.0 + (kyn.y + kyc.y)) * xc.y - kyc.y * xm.y - (gm + ge);
-            base.x = cx * xc.x + cz * z2.x + cr * rq.x;
-            base.y = cx * xc.y + cz * z2.y + cr * rq.y;
-            double2 zn;
-            zn.x = fma(-ca, fma(-kyn.x, xp.x, AXo.x), base.x);
-            zn.y = fma(-ca, fma(-kyn.y, xp.y, AXo.y), base.y);
-            const bool rowout = q >= kt0 && q < kt1;
-            if (t < M) {
-                W[t < M ? t : 0][md(ph - t, 3)] = zn;
-                if (t == M - 1 && !LAST && rowout) st2m(zoutA + (orow - t * pitch), zn, oA, oB);
-            } else if (rowout) {
-                st2m(zoutB + (orow - t * pitch), zn, oA, oB);
-                if (LAST && q >= Dd.k0 && q < Dd.k1) {
-                    if (dA) {
-                        dot0 += rq.x * zn.x;
-                        dot1 += rq.x * rq.x;
-                    }
-                    if (dB) {
-                        dot0 += rq.y * zn.y;
-                        dot1 += rq.y * rq.y;
-                    }
-                }
-            }
-        }
-    };
-    for (int kk = 0; kk < nrows; kk += P) {
-        body(std::integral_constant<int, 0>{}, kk);
-        if (kk + 1 < nrows) body(std::integral_constant<int, 1>{}, kk + 1);
-        if (kk + 2 < nrows) body(std::integral_constant<int, 2>{}, kk + 2);
-        if (kk + 3 < nrows) body(std::integral_constant<int, 3>{}, kk + 3);
-        if (kk + 4 < nrows) body(std::integral_constant<int, 4>{}, kk + 4);
-        if (kk + 5 < nrows) body(std::integral_constant<int, 5>{}, kk + 5);
-    }
-    if (LAST) {
-        double t0, t1;
-        if (grid_reduce2(dot0, dot1, a.partials, &S->ticket, &t0, &t1)) {
-            if (threadIdx.x == 0) {
-                S->red_gam = t0;
-                S->red_rr = t1;
-                if (FUSE) S->alpha_prev = alpha;
-                if (!restart) {
-                    S->it += 1;
-                    S->outer += 1;
-                }
-            }
-        }
-    } else if (FUSE) {
-        if (blockIdx.x == 0 && blockIdx.y == 0 && threadIdx.x == 0) S->alpha_prev = alpha;
-    }
-}
-
 int tb_out_cols(int M) {
     const int mr = (M + 1) & ~1;
     return kStrip - 2 * mr;
-}
-
-// 0: k_cheb_tb (LDG + shared-memory delay lines), 1: k_cheb_tma (TMA ring + register
-// delay lines), 2: k_cheb_tb6 (k_cheb_tb unrolled by the rotation period). TEA_TB_IMPL overrides (measurement knob).
-int tb_impl() {
-    static int v = [] {
-        const char *e = getenv("TEA_TB_IMPL");
-        return e ? atoi(e) : 2;
-    }();
-    return v;
 }
 
 template <int M, bool FIRST, bool FUSE, bool LAST>
@@ -960,45 +434,11 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
                       int step0, bool restart,
                       const double *rin, const double *win, double *rout, const double *zin1,
                       const double *zin2, double *zoutA, double *zoutB, const double *kx,
-                      const double *ky, const double *pin, double *u, cudaStream_t st) {
+                      const double *ky, cudaStream_t st) {
     using G = TbGeom<M>;
     const int width = R.j1 - (R.j0 & ~1);
     const int nstrips = (width + G::OW - 1) / G::OW;
     dim3 grid((nstrips + kWarps - 1) / kWarps, (R.k1 - R.k0 + ty - 1) / ty);
-    const int rs = restart ? 1 : 0;
-    if (tb_impl() == 1 || (FIRST && FUSE && u)) {
-        auto go = [&](auto kern, size_t smem, bool &attr) {
-            if (!attr) {
-                cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-                attr = true;
-            }
-            kern<<<grid, kThreads, smem, st>>>(rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky,
-                                               pin, u, a, R, Dd, ty, jlim, step0, rs);
-        };
-        if constexpr (FIRST && FUSE) {
-            if (u) {
-                static bool attr_u = false;
-                go(k_cheb_tma<M, FIRST, FUSE, LAST, true>, tma_smem_bytes<FIRST, FUSE, true>(),
-                   attr_u);
-                return;
-            }
-        }
-        static bool attr_t = false;
-        go(k_cheb_tma<M, FIRST, FUSE, LAST, false>, tma_smem_bytes<FIRST, FUSE, false>(), attr_t);
-        return;
-    }
-    if (tb_impl() == 2) {
-        constexpr size_t sm6 = tb6_smem_bytes();
-        static bool attr6 = false;
-        if (!attr6) {
-            cudaFuncSetAttribute(k_cheb_tb6<M, FIRST, FUSE, LAST>,
-                                 cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm6);
-            attr6 = true;
-        }
-        k_cheb_tb6<M, FIRST, FUSE, LAST><<<grid, kThreads, sm6, st>>>(
-            rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, a, R, Dd, ty, jlim, step0, rs);
-        return;
-    }
     constexpr size_t smem = tb_smem_bytes();
     static bool attr = false;  // per instantiation
     if (!attr) {
@@ -1007,7 +447,7 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
         attr = true;
     }
     k_cheb_tb<M, FIRST, FUSE, LAST><<<grid, kThreads, smem, st>>>(
-        rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, pin, u, a, R, Dd, ty, jlim, step0, rs);
+        rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, a, R, Dd, ty, jlim, step0, restart ? 1 : 0);
 }
 
 template <int M>
@@ -1015,11 +455,10 @@ static void tb_dispatch(const KArgs &a, const Region &R, const Region &Dd, int t
                         int step0, bool first,
                         bool fuse, bool last, bool restart, const double *rin, const double *win,
                         double *rout, const double *zin1, const double *zin2, double *zoutA,
-                        double *zoutB, const double *kx, const double *ky, const double *pin,
-                        double *u, cudaStream_t st) {
+                        double *zoutB, const double *kx, const double *ky, cudaStream_t st) {
 #define TB(F, U, L)                                                                            \
     tb_launch<M, F, U, L>(a, R, Dd, ty, jlim, step0, restart, rin, win, rout, zin1, zin2, zoutA, \
-                          zoutB, kx, ky, pin, u, st)
+                          zoutB, kx, ky, st)
     if (first) {
         if (fuse) {
             if (last) TB(true, true, true); else TB(true, true, false);
@@ -1049,22 +488,6 @@ int tb_auto_rows(int M, int width, int height) {
         switch (M) {
 #define OCC(m)                                                                                   \
     case m:                                                                                      \
-        if (tb_impl() == 2) {                                                                    \
-            const size_t sm6 = tb6_smem_bytes();                                                 \
-            cudaFuncSetAttribute(k_cheb_tb6<m, false, false, true>,                              \
-                                 cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm6);         \
-            e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(                                   \
-                &per, k_cheb_tb6<m, false, false, true>, kThreads, sm6);                         \
-            break;                                                                               \
-        }                                                                                        \
-        if (tb_impl() == 1) {                                                                    \
-            const size_t sm2 = tma_smem_bytes<false, false, false>();                            \
-            cudaFuncSetAttribute(k_cheb_tma<m, false, false, true, false>,                       \
-                                 cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm2);         \
-            e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(                                   \
-                &per, k_cheb_tma<m, false, false, true, false>, kThreads, sm2);                  \
-            break;                                                                               \
-        }                                                                                        \
         cudaFuncSetAttribute(k_cheb_tb<m, false, false, true>,                                   \
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);            \
         e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per, k_cheb_tb<m, false, false, true>, \
@@ -1105,13 +528,13 @@ void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, in
                     bool first, bool fuse, bool last, bool restart, const double *rin,
                     const double *win, double *rout, const double *zin1, const double *zin2,
                     double *zoutA, double *zoutB, const double *kx, const double *ky,
-                    const double *pin, double *u, cudaStream_t st) {
+                    cudaStream_t st) {
     switch (M) {
-        case 1: tb_dispatch<1>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, pin, u, st); break;
-        case 2: tb_dispatch<2>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, pin, u, st); break;
-        case 3: tb_dispatch<3>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, pin, u, st); break;
-        case 4: tb_dispatch<4>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, pin, u, st); break;
-        default: tb_dispatch<5>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, pin, u, st); break;
+        case 1: tb_dispatch<1>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
+        case 2: tb_dispatch<2>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
+        case 3: tb_dispatch<3>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
+        case 4: tb_dispatch<4>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
+        default: tb_dispatch<5>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
     }
 }
 

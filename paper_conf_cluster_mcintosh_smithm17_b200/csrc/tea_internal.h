@@ -104,7 +104,6 @@ void launch_init_fields3(const KArgs &a, const double *rho, const double *en, do
 void launch_residual(const KArgs &a, const Launch &L, const Region &R, const double *u,
                      const double *kx, const double *ky, double *u0, double *r,
                      cudaStream_t st);
-// u == nullptr: no lazy u += alpha_prev p_old (the caller's next kernel applies alpha)
 void launch_spmv(const KArgs &a, const Launch &L, const Region &R, const double *src,
                  const double *pin, double *pout, double *w, double *u, const double *kx,
                  const double *ky, cudaStream_t st);
@@ -156,8 +155,7 @@ void launch_cg1_update(const KArgs &a, const Launch &L, const Region &R, const d
 void launch_cg1_w(const KArgs &a, const Launch &L, const Region &R, const double *r, double *w,
                   const double *kx, const double *ky, cudaStream_t st);
 
-// Temporally blocked Chebyshev passes (tea_cheb_tb.cu). fuse (first pass): r_out = r_in -
-// alpha w and u += alpha pin on the owned cells.
+// Temporally blocked Chebyshev passes (tea_cheb_tb.cu).
 constexpr int kTbMaxSteps = 5;
 int tb_out_cols(int M);
 int tb_ctas(int M, int width, int height, int ty);
@@ -169,6 +167,6 @@ void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, in
                     int step0, bool first, bool fuse, bool last, bool restart, const double *rin,
                     const double *win, double *rout, const double *zin1, const double *zin2,
                     double *zoutA, double *zoutB, const double *kx, const double *ky,
-                    const double *pin, double *u, cudaStream_t st);
+                    cudaStream_t st);
 
 }  // namespace tea
