@@ -568,6 +568,10 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
             int ty = c->opts.tb_rows > 0 ? c->opts.tb_rows : 0;
             // tall tiles keep the 2M-row pipeline fill small; whole waves (tb_auto_rows)
             if (ty <= 0) ty = tb_auto_rows(M, R.j1 - R.j0, R.k1 - R.k0);
+            // two reduction partials per CTA must fit the block's scratch
+            while (ty < R.k1 - R.k0 &&
+                   2 * (size_t)tb_ctas(M, R.j1 - R.j0, R.k1 - R.k0, ty) > b.L.partials_cap)
+                ty *= 2;
             int streams = first ? (fu ? 4 : 3) : 5;     // reads
             streams += (fu ? 1 : 0) + (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})
             const int kid = last ? TEA_K_TB_LAST : (first ? TEA_K_TB_FIRST : TEA_K_TB_MID);

@@ -27,6 +27,15 @@
 
 namespace tea {
 
+#ifndef TEA_TB_WARPS
+#define TEA_TB_WARPS 4
+#endif
+// warps per CTA of the fused passes (each warp marches its own strip; CTAs only share the
+// grid reduction). Smaller CTAs pack registers tighter: 138 registers allow 14 warps per SM
+// but only 3 CTAs of 4 warps.
+constexpr int kTbW = TEA_TB_WARPS;
+constexpr int kTbT = 32 * kTbW;
+
 // Chebyshev coefficients of the fused passes live in constant memory (one slot per
 // context): uniform per-step scalars then cost LDC through the constant cache instead
 // of shared-memory wavefronts on the L1TEX pipe the passes are bound by.
@@ -81,7 +90,7 @@ __device__ __forceinline__ double wsum(double v) {
 // Deterministic two-value grid reduction (same scheme as tea_kernels.cu).
 __device__ bool grid_reduce2(double v0, double v1, double *partials, unsigned *ticket,
                              double *out0, double *out1) {
-    __shared__ double sh[2][kWarps];
+    __shared__ double sh[2][kTbW];
     __shared__ bool last;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const int nblk = gridDim.x * gridDim.y * gridDim.z;
@@ -95,7 +104,7 @@ __device__ bool grid_reduce2(double v0, double v1, double *partials, unsigned *t
     __syncthreads();
     if (threadIdx.x == 0) {
         double s0 = 0.0, s1 = 0.0;
-        for (int w = 0; w < kWarps; ++w) {
+        for (int w = 0; w < kTbW; ++w) {
             s0 += sh[0][w];
             s1 += sh[1][w];
         }
@@ -111,13 +120,13 @@ __device__ bool grid_reduce2(double v0, double v1, double *partials, unsigned *t
 #pragma unroll
     for (int i = 0; i < 2; ++i) {
         double s = 0.0;
-        for (int b = threadIdx.x; b < nblk; b += kThreads) s += __ldcg(partials + i * nblk + b);
+        for (int b = threadIdx.x; b < nblk; b += kTbT) s += __ldcg(partials + i * nblk + b);
         s = wsum(s);
         __syncthreads();
         if (lane == 0) sh[i][warp] = s;
         __syncthreads();
         double a = 0.0;
-        for (int w = 0; w < kWarps; ++w) a += sh[i][w];
+        for (int w = 0; w < kTbW; ++w) a += sh[i][w];
         t[i] = a;
     }
     *out0 = t[0];
@@ -148,7 +157,7 @@ constexpr int kTbUnroll = TEA_TB_UNROLL;  // measured: 2 (step t+1 of row k over
 
 // dynamic shared memory of a pass: the Kx, Ky, r delay rings (depth 8, one double2 per
 // thread and row)
-constexpr size_t tb_smem_bytes() { return sizeof(double2) * 3 * 8 * kThreads; }
+constexpr size_t tb_smem_bytes() { return sizeof(double2) * 3 * 8 * kTbT; }
 
 template <int M>
 struct TbGeom {
@@ -173,7 +182,7 @@ struct TbGeom {
 #endif
 #define TB_REG_R (TEA_TB_REGLINES >= 1)
 template <int M, bool FIRST, bool FUSE, bool LAST>
-__global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
+__global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     k_cheb_tb(const double *__restrict__ rin, const double *__restrict__ win,
               double *__restrict__ rout, const double *__restrict__ zin1,
               const double *__restrict__ zin2, double *__restrict__ zoutA,
@@ -184,9 +193,9 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
     constexpr int D = G::D;
     static_assert(M <= 6, "delay lines hold M+2 rows");
     extern __shared__ double2 tb_smem[];
-    double2(*ringKx)[kThreads] = reinterpret_cast<double2(*)[kThreads]>(tb_smem);
-    double2(*ringKy)[kThreads] = ringKx + D;
-    double2(*ringR)[kThreads] = ringKy + D;
+    double2(*ringKx)[kTbT] = reinterpret_cast<double2(*)[kTbT]>(tb_smem);
+    double2(*ringKy)[kTbT] = ringKx + D;
+    double2(*ringR)[kTbT] = ringKy + D;
     const double(*coef)[kMaxS] = c_tb_coef[a.coef_slot];
 
     Scalars *S = a.S;
@@ -219,7 +228,7 @@ __global__ void __launch_bounds__(kThreads, TEA_TB_MINB)
 
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5, tid = threadIdx.x;
     (void)tid;
-    const int strip = blockIdx.x * kWarps + warp;
+    const int strip = blockIdx.x * kTbW + warp;
     // strips tile the output region R (which may reach into the halo on sides with a
     // neighbour block: extended bounds); first strip starts MR before it
     const int jA = (R.j0 & ~1) - G::MR + strip * G::OW + 2 * lane;
@@ -438,7 +447,7 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
     using G = TbGeom<M>;
     const int width = R.j1 - (R.j0 & ~1);
     const int nstrips = (width + G::OW - 1) / G::OW;
-    dim3 grid((nstrips + kWarps - 1) / kWarps, (R.k1 - R.k0 + ty - 1) / ty);
+    dim3 grid((nstrips + kTbW - 1) / kTbW, (R.k1 - R.k0 + ty - 1) / ty);
     constexpr size_t smem = tb_smem_bytes();
     static bool attr = false;  // per instantiation
     if (!attr) {
@@ -446,7 +455,7 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         attr = true;
     }
-    k_cheb_tb<M, FIRST, FUSE, LAST><<<grid, kThreads, smem, st>>>(
+    k_cheb_tb<M, FIRST, FUSE, LAST><<<grid, kTbT, smem, st>>>(
         rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, a, R, Dd, ty, jlim, step0, restart ? 1 : 0);
 }
 
@@ -491,7 +500,7 @@ int tb_auto_rows(int M, int width, int height) {
         cudaFuncSetAttribute(k_cheb_tb<m, false, false, true>,                                   \
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);            \
         e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per, k_cheb_tb<m, false, false, true>, \
-                                                          kThreads, smem);                       \
+                                                          kTbT, smem);                       \
         break;
             OCC(1) OCC(2) OCC(3) OCC(4) OCC(5)
 #undef OCC
@@ -500,7 +509,7 @@ int tb_auto_rows(int M, int width, int height) {
         slots[M] = nsm * per;
     }
     const int ow = tb_out_cols(M);
-    const int gx = ((width + ow - 1) / ow + kWarps - 1) / kWarps;
+    const int gx = ((width + ow - 1) / ow + kTbW - 1) / kTbW;
     int best = height, bestc = 0x7fffffff;
     for (int w = 1; w <= 256; ++w) {
         const int tiles = (int)((long long)slots[M] * w / gx);
@@ -520,7 +529,7 @@ int tb_auto_rows(int M, int width, int height) {
 int tb_ctas(int M, int width, int height, int ty) {
     const int ow = tb_out_cols(M);
     const int nstrips = (width + ow - 1) / ow;
-    return ((nstrips + kWarps - 1) / kWarps) * ((height + ty - 1) / ty);
+    return ((nstrips + kTbW - 1) / kTbW) * ((height + ty - 1) / ty);
 }
 
 void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, int ty, int jlim,
