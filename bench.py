@@ -285,7 +285,8 @@ def run_gpu(args):
               "cg1": tea.CG1, "jacobi": tea.JACOBI, "cheby": tea.CHEBY}[args.method]
     cells = args.n * args.n * max(args.nz, 1)
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
-                tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode)
+                tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode,
+                persist=args.persist)
     stream = t.stream
 
     def solve():
@@ -426,6 +427,9 @@ def main():
                     help="PXxPY: run the px x py decomposition inside ONE process on one GPU "
                          "(the multi-GPU code path with device-copy halos instead of NCCL)")
     ap.add_argument("--tile-rows", type=int, default=0)
+    ap.add_argument("--persist", type=int, default=0,
+                    help="whole solve in one cooperative launch: 1 on, 0 (auto) or -1 off "
+                         "(tea_opts.persist)")
     ap.add_argument("--tb-steps", type=int, default=0,
                     help="Chebyshev steps per fused HBM pass (0 auto=4, 1 = per-step kernels)")
     ap.add_argument("--loop-mode", type=int, default=0,

@@ -31,7 +31,7 @@
 extern "C" {
 #endif
 
-#define TEA_ABI_VERSION 1
+#define TEA_ABI_VERSION 2
 
 typedef enum {
     TEA_OK = 0,
@@ -105,6 +105,11 @@ typedef struct {
                                powers, single block only): 0 = auto, 1 = one kernel
                                per step, 2..5 = at most that many            [0 = 4] */
     int tb_rows;            /* output rows per CTA tile of the fused passes, 0 = auto */
+    int persist;            /* whole solve in ONE cooperative launch (grid-wide barriers
+                               between the phases; single 2D block, CG / CPPCG, one
+                               process, loop_mode 0): 1 = on; 0 (auto) and -1 = off:
+                               measured slower than the graph path at every size
+                               tried                        [0] */
 } tea_opts;
 
 /* Per-solve statistics. */
@@ -130,6 +135,7 @@ enum {
     TEA_K_BJ,                                     /* block-Jacobi update + strip solves  */
     TEA_K_CG1, TEA_K_CG1W,                        /* single-reduction CG: fused / A r    */
     TEA_K_STAT,                                   /* Jacobi / Chebyshev iteration        */
+    TEA_K_PERSIST,                                /* whole solve, one cooperative launch */
     TEA_K_COUNT
 };
 

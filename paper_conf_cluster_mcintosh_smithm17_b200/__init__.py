@@ -25,7 +25,7 @@ OK, NOT_CONVERGED = 0, 1
 ERR_ARG, ERR_CUDA, ERR_NCCL, ERR_BREAKDOWN, ERR_STATE = -1, -2, -3, -4, -5
 KERNELS = ["init", "residual", "spmv", "update", "cheb_first", "cheb_step", "cheb_last", "eig",
            "pack", "unpack", "scalar", "tb_first", "tb_mid", "tb_last", "bj", "cg1",
-           "cg1_w", "stat"]
+           "cg1_w", "stat", "persist"]
 SYMBOLS = ["tea_version", "tea_abi_version", "tea_get_nccl_id", "tea_workspace_bytes", "tea_init",
            "tea_solve", "tea_fetch", "tea_set_u", "tea_kernel_times", "tea_launch_count",
            "tea_finalize", "tea_last_error", "tea_block_extent", "tea_cheb_schedule"]
@@ -43,6 +43,9 @@ class Mesh(C.Structure):
                 ("zmin", C.c_double), ("zmax", C.c_double)]
 
 
+ABI_VERSION = 2  # include/tea.h TEA_ABI_VERSION (tea_opts layout)
+
+
 class Dist(C.Structure):
     _fields_ = [("rank", C.c_int), ("nranks", C.c_int), ("px", C.c_int), ("py", C.c_int),
                 ("halo_depth", C.c_int), ("nccl_id", C.c_void_p)]
@@ -52,7 +55,7 @@ class Opts(C.Structure):
     _fields_ = [("presteps", C.c_int), ("eig_margin_lo", C.c_double),
                 ("eig_margin_hi", C.c_double), ("mean_mode", C.c_int), ("loop_mode", C.c_int),
                 ("check_interval", C.c_int), ("profile", C.c_int), ("tile_rows", C.c_int),
-                ("tb_steps", C.c_int), ("tb_rows", C.c_int)]
+                ("tb_steps", C.c_int), ("tb_rows", C.c_int), ("persist", C.c_int)]
 
 
 class Stats(C.Structure):
@@ -85,6 +88,9 @@ def lib(build_if_needed: bool = True):
     vp, i, d = C.c_void_p, C.c_int, C.c_double
     L.tea_version.restype = C.c_char_p
     L.tea_abi_version.restype = i
+    if L.tea_abi_version() != ABI_VERSION:
+        raise ImportError(f"{path}: ABI version {L.tea_abi_version()} != {ABI_VERSION} "
+                          "(stale build; run __graft_entry__.build())")
     L.tea_get_nccl_id.argtypes = [vp]
     L.tea_workspace_bytes.argtypes = [C.POINTER(Mesh), C.POINTER(Dist), C.POINTER(C.c_size_t)]
     L.tea_init.argtypes = [C.POINTER(vp), C.POINTER(Mesh), vp, vp, d, C.POINTER(Dist),
@@ -173,8 +179,8 @@ class Tea:
     def __init__(self, mesh: Mesh, density, energy, dt: float, dist: dict | None = None,
                  presteps: int = 30, eig_margins=(0.95, 1.05), mean_mode: int = 0,
                  loop_mode: int = 0, check_interval: int = 0, profile: bool = False,
-                 tile_rows: int = 0, tb_steps: int = 0, tb_rows: int = 0, device=None,
-                 stream=None):
+                 tile_rows: int = 0, tb_steps: int = 0, tb_rows: int = 0, persist: int = 0,
+                 device=None, stream=None):
         import torch
         if not torch.cuda.is_available():
             raise RuntimeError("paper_conf_cluster_mcintosh_smithm17_b200 needs a CUDA device "
@@ -194,7 +200,8 @@ class Tea:
                               dist.get("py", 1), dist.get("halo_depth", 1),
                               C.cast(self._nccl_id, C.c_void_p) if self._nccl_id else None)
         self.opts = Opts(presteps, eig_margins[0], eig_margins[1], mean_mode, loop_mode,
-                         check_interval, 1 if profile else 0, tile_rows, tb_steps, tb_rows)
+                         check_interval, 1 if profile else 0, tile_rows, tb_steps, tb_rows,
+                         persist)
         with torch.cuda.device(self.device):
             nbytes = workspace_bytes(mesh, self._dist)
             self.workspace = torch.empty(nbytes, dtype=torch.uint8, device=self.device)

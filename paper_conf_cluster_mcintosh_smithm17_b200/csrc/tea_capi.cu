@@ -809,6 +809,44 @@ tea_status map_status(int ds, bool maxed) {
     }
 }
 
+// Whole solve in one cooperative launch (k_persist): one 2D block in one process, CG or
+// CPPCG, device-loop mode, no per-kernel profiling; opt-in (tea_opts.persist = 1): the
+// grid barriers cost more than graph kernel boundaries at every size measured
+// (profiles/r01f_persist.txt).
+bool use_persist(const tea_ctx *c, tea_method method) {
+    if (c->opts.persist != 1) return false;
+    if (method != TEA_CG && method != TEA_CPPCG) return false;
+    if (c->px * c->py != 1 || c->nranks != 1 || is3d(c) || c->profiling) return false;
+    return c->opts.loop_mode == 0;
+}
+
+void solve_persist(tea_ctx *c, int s, bool two_phase) {
+    BlockCtx &b = c->blocks[0];
+    PersistArgs P{};
+    P.a = kargs(c, b);
+    P.R = b.owned();
+    const Launch L = plan_st(c, b, P.R);
+    P.jstart = L.jstart;
+    P.ty = L.ty;
+    P.gx = (int)L.grid.x;
+    P.ntiles = (int)(L.grid.x * L.grid.y);
+    P.s = s;
+    P.two_phase = two_phase ? 1 : 0;
+    P.kx = b.f[F_KX];
+    P.ky = b.f[F_KY];
+    P.u0 = b.f[F_U0];
+    P.u = b.f[F_U];
+    P.w = b.f[F_W];
+    P.r[0] = b.f[F_R0];
+    P.r[1] = b.f[F_R1];
+    P.p[0] = b.f[F_P0];
+    P.p[1] = b.f[F_P1];
+    for (int i = 0; i < 3; ++i) P.z[i] = b.f[F_Z0 + i];
+    const int ctas = persist_ctas(P.ntiles);
+    K(c, TEA_K_PERSIST, 0.0, [&] { CK(launch_persist(P, ctas, c->stream)); });
+    read_state(c);
+}
+
 tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, int s,
                       tea_stats *st) {
     if (c->failed) fail(TEA_ERR_STATE, "context already failed: %s", c->err.c_str());
@@ -833,6 +871,14 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
             launch_scalars(kargs(c, b), SC_BEGIN, eps, lim1, max_iters, c->opts.eig_margin_lo,
                            c->opts.eig_margin_hi, c->stream);
         });
+    const bool persist = use_persist(c, method);
+    int ds = DS_RUNNING;
+    bool phase2 = false;
+    if (persist) {
+        solve_persist(c, s, two_phase);
+        ds = c->hS->status;
+        phase2 = two_phase && c->hS->presteps > 0;
+    } else {
     exchange(c, X_U1, {F_U});
     for (auto &b : c->blocks) {
         Region R = b.owned();
@@ -884,14 +930,14 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         else
             run_loop(c, 1, lim1, [&](int par, bool sc) { body_cg(c, par, sc); });
     }
-    int ds = c->hS->status;
+    ds = c->hS->status;
     if (method == TEA_JACOBI) {  // the final iterate is in Z0 after an odd count
         if (c->hS->it % 2 == 1)
             for (auto &b : c->blocks)
                 CK(cudaMemcpyAsync(field_base(b, F_U), field_base(b, F_Z0), b.L.field_bytes,
                                    cudaMemcpyDeviceToDevice, c->stream));
     }
-    bool phase2 = two_phase && ds == DS_LIMIT && c->hS->it < max_iters;
+    phase2 = two_phase && ds == DS_LIMIT && c->hS->it < max_iters;
     if (phase2 && method == TEA_CHEBY) {
         for (auto &b : c->blocks)
             K(c, TEA_K_EIG, 0.0, [&] { launch_eig_setup(kargs(c, b), 1, c->stream); });
@@ -919,6 +965,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         }
         ds = c->hS->status;
     }
+    }  // !persist
     CK(cudaEventRecord(c->ev_t1, c->stream));
     CK(cudaEventRecord(c->ev_in, c->stream));
     CK(cudaStreamWaitEvent(c->user_stream, c->ev_in, 0));
@@ -1066,6 +1113,7 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
             if (o.eig_margin_hi == 0.0) o.eig_margin_hi = 1.05;
         }
         if (o.loop_mode < 0 || o.loop_mode > 2) fail(TEA_ERR_ARG, "bad loop_mode");
+        if (o.persist < -1 || o.persist > 1) fail(TEA_ERR_ARG, "bad persist");
         // NCCL kernels inside a WHILE-conditional graph body are not a supported
         // capture target: multi-process runs use chunked graphs (same kernels).
         if (nranks > 1 && o.loop_mode == 0) o.loop_mode = 1;

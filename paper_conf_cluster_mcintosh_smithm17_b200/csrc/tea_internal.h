@@ -169,4 +169,18 @@ void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, in
                     double *zoutA, double *zoutB, const double *kx, const double *ky,
                     cudaStream_t st);
 
+// Persistent single-launch CG / CPPCG solve of one 2D block (tea_kernels.cu, k_persist):
+// phases separated by grid-wide barriers of a cooperative launch.
+struct PersistArgs {
+    KArgs a;
+    Region R;  // owned cells
+    int jstart, ty, gx, ntiles;  // stencil tiling (plan_stencil)
+    int s, two_phase;            // inner steps; 1 = CPPCG (presteps, eigen-estimate, PCG)
+    const double *kx, *ky;
+    double *u0, *u, *w;
+    double *r[2], *p[2], *z[3];
+};
+int persist_ctas(int ntiles);  // co-resident CTAs for a tiling of ntiles (<= ntiles)
+cudaError_t launch_persist(const PersistArgs &P, int ctas, cudaStream_t st);
+
 }  // namespace tea

@@ -51,7 +51,7 @@ def test_sm100a_sass():
 
 def test_version(L):
     assert "sm_100a" in tea.version()
-    assert L.tea_abi_version() == 1
+    assert L.tea_abi_version() == 2
 
 
 @pytest.mark.parametrize("nx,ny,px,py", [(4096, 4096, 2, 4), (1000, 777, 3, 2), (17, 5, 4, 1),

@@ -526,3 +526,61 @@ def test_fused_passes_blocks_fixed_iterations(tea, ora):
                       **kw)
     assert st[0]["iterations"] == 34
     assert field_err(u_g, u_o, "random") <= 1e-12
+
+
+# ---------------------------------------------------------------- persistent solver
+# tea_opts.persist = 1: the whole solve in ONE cooperative launch (k_persist, grid-wide
+# barriers between the phases). Same device bodies as the graph path.
+@pytest.mark.parametrize("kind,nx,ny", SHAPES[:7])
+@pytest.mark.parametrize("k", [1, 7])
+def test_persist_fixed_cg_iterations(tea, ora, kind, nx, ny, k):
+    deck = deck_of(kind, nx, ny, seed=nx + ny, dt=0.04)
+    u_o, st_o, _ = ora.run(deck, steps=1, method=0, eps=0.0, max_iters=k)
+    u_g, st_g = gpu_run(tea, deck, method=0, eps=0.0, max_iters=k, persist=1)
+    assert st_g[0]["iterations"] == st_o[0]["iterations"] == k
+    assert st_g[0]["ret"] == 1
+    assert field_err(u_g, u_o, kind) <= 1e-12
+
+
+@pytest.mark.parametrize("kind,nx,ny", [("pipe", 128, 128), ("random", 300, 200),
+                                        ("random", 257, 65)])
+@pytest.mark.parametrize("method", [0, 1])
+def test_persist_converged(tea, ora, kind, nx, ny, method):
+    deck = deck_of(kind, nx, ny, seed=3, dt=0.004)
+    kw = dict(method=method, eps=1e-13, max_iters=20000, inner_steps=6)
+    u_o, st_o, s_o = ora.run(deck, steps=1, **kw)
+    u_p, st_p = gpu_run(tea, deck, persist=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, persist=-1, **kw)
+    assert s_o[0] == 0 and st_p[0]["ret"] == 0
+    assert abs(st_p[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert abs(st_p[0]["iterations"] - st_g[0]["iterations"]) <= 1
+    assert field_err(u_p, u_o, kind) <= 1e-10
+    assert field_err(u_p, u_g, kind) <= 1e-11
+    if method == 1 and st_o[0]["outer"] > 0:
+        assert st_p[0]["presteps"] == st_o[0]["presteps"]
+        assert st_p[0]["eig_max"] == pytest.approx(st_o[0]["eig_max"], rel=1e-9)
+
+
+def test_persist_config1_10_steps(tea, ora):
+    """BASELINE configs[0] (128^2 CG, 10 timesteps, eps 1e-15) through one launch per step."""
+    deck = deck_of("pipe", 128, 128)
+    kw = dict(method=0, eps=1e-15, max_iters=10000)
+    u_o, st_o, _ = ora.run(deck, steps=10, **kw)
+    u_g, st_g = gpu_run(tea, deck, steps=10, persist=1, **kw)
+    for a, b in zip(st_g, st_o):
+        assert abs(a["iterations"] - b["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+
+
+@pytest.mark.parametrize("tile_rows", [1, 3, 8])
+def test_persist_many_tiles_per_cta(tea, tile_rows):
+    """1024^2 with short tiles: more tiles than co-resident CTAs, so each CTA walks
+    several tiles per phase; 30 presteps + 3 outer against the graph path."""
+    from paper_conf_cluster_mcintosh_smithm17_b200 import inputs
+    deck = inputs.crooked_pipe(1024)
+    kw = dict(method=1, eps=0.0, max_iters=33, inner_steps=10, tile_rows=tile_rows)
+    u_p, st_p = gpu_run(tea, deck, persist=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, persist=-1, **kw)
+    assert st_p[0]["iterations"] == st_g[0]["iterations"] == 33
+    assert st_p[0]["outer"] == st_g[0]["outer"] == 3
+    assert rel_err(u_p, u_g) <= 1e-12
