@@ -107,10 +107,13 @@ typedef struct {
     int tb_rows;            /* output rows per CTA tile of the fused passes, 0 = auto */
     int persist;            /* whole solve in ONE cooperative launch (grid-wide barriers
                                between the phases; single 2D block, CG / CPPCG, one
-                               process, loop_mode 0): 1 = on; 0 (auto) and -1 = off:
-                               measured slower than the graph path at every size
-                               tried                        [0] */
+                               process, loop_mode 0): 1 = on, -1 = off, 0 = auto:
+                               on for CG blocks <= TEA_PERSIST_AUTO_CG cells and
+                               CPPCG blocks <= TEA_PERSIST_AUTO_CPPCG cells, where it
+                               measured faster              [0] */
 } tea_opts;
+#define TEA_PERSIST_AUTO_CG (1024.0 * 1024.0)
+#define TEA_PERSIST_AUTO_CPPCG (512.0 * 512.0)
 
 /* Per-solve statistics. */
 typedef struct {

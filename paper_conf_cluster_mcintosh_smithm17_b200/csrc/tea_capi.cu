@@ -81,6 +81,7 @@ BlockLayout layout_block(const tea_mesh &m, int px, int py, int d, int b) {
     off += round_up(sizeof(Scalars), 256);
     L.partials_cap = 2 * (size_t)std::max(max_ctas(L.bx + 2 * d + 2, L.by + 2 * d + 2),
                                           L.nz > 1 ? max_ctas3(L.bx, L.by, L.nz) : 0);
+    L.partials_cap = std::max(L.partials_cap, (size_t)6 * 1024);  // k_persist: 2 x 3 x CTAs
     L.partials_off = off;
     off += round_up(L.partials_cap * sizeof(double), 256);
     L.has_nbr = (px * py > 1);
@@ -810,14 +811,17 @@ tea_status map_status(int ds, bool maxed) {
 }
 
 // Whole solve in one cooperative launch (k_persist): one 2D block in one process, CG or
-// CPPCG, device-loop mode, no per-kernel profiling; opt-in (tea_opts.persist = 1): the
-// grid barriers cost more than graph kernel boundaries at every size measured
-// (profiles/r01f_persist.txt).
+// CPPCG, device-loop mode, no per-kernel profiling. Auto (persist = 0): where it measured
+// faster than the graph path (profiles/r01f_persist.txt): CG up to 1024^2 cells, CPPCG up
+// to 512^2 (beyond, the per-phase barrier no longer hides behind the tile work).
 bool use_persist(const tea_ctx *c, tea_method method) {
-    if (c->opts.persist != 1) return false;
+    if (c->opts.persist < 0) return false;
     if (method != TEA_CG && method != TEA_CPPCG) return false;
     if (c->px * c->py != 1 || c->nranks != 1 || is3d(c) || c->profiling) return false;
-    return c->opts.loop_mode == 0;
+    if (c->opts.loop_mode != 0) return false;
+    if (c->opts.persist == 1) return true;
+    const double cells = (double)c->blocks[0].L.bx * c->blocks[0].L.by;
+    return cells <= (method == TEA_CG ? TEA_PERSIST_AUTO_CG : TEA_PERSIST_AUTO_CPPCG);
 }
 
 void solve_persist(tea_ctx *c, int s, bool two_phase) {
@@ -825,7 +829,16 @@ void solve_persist(tea_ctx *c, int s, bool two_phase) {
     PersistArgs P{};
     P.a = kargs(c, b);
     P.R = b.owned();
-    const Launch L = plan_st(c, b, P.R);
+    Launch L = plan_st(c, b, P.R);
+    if (c->opts.tile_rows <= 0) {
+        // one tile per resident CTA: the phase time is the slowest CTA's tile chain, so
+        // the tallest tiles that still fit the co-resident grid in ONE round
+        const int cap = std::min(persist_ctas(1 << 30), (int)(b.L.partials_cap / 6));
+        const int gx = (int)L.grid.x, height = P.R.k1 - P.R.k0;
+        const int gy = std::max(1, cap / gx);
+        const int ty = std::max(1, (height + gy - 1) / gy);
+        L = plan_stencil(P.R, ty, 0);
+    }
     P.jstart = L.jstart;
     P.ty = L.ty;
     P.gx = (int)L.grid.x;
@@ -842,7 +855,8 @@ void solve_persist(tea_ctx *c, int s, bool two_phase) {
     P.p[0] = b.f[F_P0];
     P.p[1] = b.f[F_P1];
     for (int i = 0; i < 3; ++i) P.z[i] = b.f[F_Z0 + i];
-    const int ctas = persist_ctas(P.ntiles);
+    P.part = b.partials;
+    const int ctas = std::min(persist_ctas(P.ntiles), (int)(b.L.partials_cap / 6));
     K(c, TEA_K_PERSIST, 0.0, [&] { CK(launch_persist(P, ctas, c->stream)); });
     read_state(c);
 }

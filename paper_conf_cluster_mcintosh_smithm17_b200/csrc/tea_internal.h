@@ -179,6 +179,7 @@ struct PersistArgs {
     const double *kx, *ky;
     double *u0, *u, *w;
     double *r[2], *p[2], *z[3];
+    double *part;  // 2 x 3 x gridDim.x reduction partials
 };
 int persist_ctas(int ntiles);  // co-resident CTAs for a tiling of ntiles (<= ntiles)
 cudaError_t launch_persist(const PersistArgs &P, int ctas, cudaStream_t st);

@@ -70,12 +70,14 @@ SHAPES = [("pipe", 128, 128), ("random", 300, 200), ("random", 1000, 777), ("ran
 
 @pytest.mark.parametrize("kind,nx,ny", SHAPES)
 @pytest.mark.parametrize("k", [1, 2, 7])
-def test_fixed_cg_iterations(tea, ora, kind, nx, ny, k):
+@pytest.mark.parametrize("persist", [0, -1])
+def test_fixed_cg_iterations(tea, ora, kind, nx, ny, k, persist):
     """k CG iterations with eps = 0: exercises residual, spmv (+ lazy u update),
-    update and the finalize path on ragged shapes."""
+    update and the finalize path on ragged shapes (persist 0: the auto choice -- the
+    persistent solver at these sizes; -1: the graph path)."""
     deck = deck_of(kind, nx, ny, seed=nx + ny, dt=0.04)
     u_o, st_o, _ = ora.run(deck, steps=1, method=0, eps=0.0, max_iters=k)
-    u_g, st_g = gpu_run(tea, deck, method=0, eps=0.0, max_iters=k)
+    u_g, st_g = gpu_run(tea, deck, method=0, eps=0.0, max_iters=k, persist=persist)
     assert st_g[0]["iterations"] == st_o[0]["iterations"] == k
     assert st_g[0]["ret"] == 1  # TEA_NOT_CONVERGED
     assert field_err(u_g, u_o, kind) <= 1e-12
@@ -84,14 +86,15 @@ def test_fixed_cg_iterations(tea, ora, kind, nx, ny, k):
 
 @pytest.mark.parametrize("kind,nx,ny", SHAPES[:5])
 @pytest.mark.parametrize("method", [0, 1])
-def test_converged_solve(tea, ora, kind, nx, ny, method):
+@pytest.mark.parametrize("persist", [0, -1])
+def test_converged_solve(tea, ora, kind, nx, ny, method, persist):
     # dt = 0.004 (the deck's): kappa ~ 1e3-1e4. At kappa ~ 1e6 (dt = 0.4, 3700 CG
     # iterations) CG's finite-precision iteration count drifts by ~10 between any two
     # summation orders, so +-2 is not a meaningful bar there.
     deck = deck_of(kind, nx, ny, seed=3, dt=0.004)
     kw = dict(method=method, eps=1e-13, max_iters=20000, inner_steps=6)
     u_o, st_o, s_o = ora.run(deck, steps=1, **kw)
-    u_g, st_g = gpu_run(tea, deck, **kw)
+    u_g, st_g = gpu_run(tea, deck, persist=persist, **kw)
     assert s_o[0] == 0 and st_g[0]["ret"] == 0
     assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
     assert field_err(u_g, u_o, kind) <= 1e-10
@@ -102,11 +105,12 @@ def test_converged_solve(tea, ora, kind, nx, ny, method):
 
 
 def test_config1_pipe128_cg_10_steps(tea, ora):
-    """BASELINE.json configs[0]: 128x128, CG, fp64, 10 timesteps, eps = 1e-15."""
+    """BASELINE.json configs[0]: 128x128, CG, fp64, 10 timesteps, eps = 1e-15 (graph path;
+    the persistent solver: test_persist_config1_10_steps)."""
     deck = deck_of("pipe", 128, 128)
     kw = dict(method=0, eps=1e-15, max_iters=10000)
     u_o, st_o, _ = ora.run(deck, steps=10, **kw)
-    u_g, st_g = gpu_run(tea, deck, steps=10, **kw)
+    u_g, st_g = gpu_run(tea, deck, steps=10, persist=-1, **kw)
     for a, b in zip(st_g, st_o):
         assert abs(a["iterations"] - b["iterations"]) <= 2
     assert rel_err(u_g, u_o) <= 1e-10

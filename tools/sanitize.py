@@ -17,13 +17,19 @@ def main():
         (inputs.crooked_pipe(96, 70), None, dict(tb_steps=5)),      # fused passes forced on
         (inputs.random_fields(67, 45, 3), dict(px=2, py=2, halo_depth=3, nranks=1), {}),
         (inputs.crooked_pipe3(20, 18, 9), None, {}),
+        # persistent solver (one cooperative launch; needs the device-loop mode)
+        (inputs.crooked_pipe(96, 70), None, dict(persist=1, loop_mode=0)),
+        (inputs.random_fields(300, 41, 5), None, dict(persist=1, loop_mode=0, tile_rows=1)),
     ]
     for deck, dist, kw in cases:
         for method in (0, 1, 2, 3, 4, 5):
             if getattr(deck, "nz", 1) > 1 and method == 2:
                 continue
+            if kw.get("persist") and method > 1:
+                continue
+            kw = dict(dict(loop_mode=2, check_interval=4), **kw)
             t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist,
-                        loop_mode=2, check_interval=4, presteps=10, **kw)
+                        presteps=10, **kw)
             r = t.solve(method, 1e-10, 60, 4, raise_on_error=False)
             t.fetch()
             t.close()
