@@ -35,6 +35,17 @@ namespace tea {
 // but only 3 CTAs of 4 warps.
 constexpr int kTbW = TEA_TB_WARPS;
 constexpr int kTbT = 32 * kTbW;
+#ifndef TEA_TB_TMEM
+#define TEA_TB_TMEM 1  // Kx, Ky, r delay lines in tensor memory (see tm_st12)
+#endif
+#ifndef TEA_TB_CPA
+#define TEA_TB_CPA 4  // rows of cp.async input staging ahead of the march (0: one register row)
+#endif
+#define TB_CPA (TEA_TB_CPA > 0)
+#if TB_CPA && !TEA_TB_TMEM
+#error "TEA_TB_CPA stages rows in the shared memory the rings would use: needs TEA_TB_TMEM"
+#endif
+constexpr int kTbNS = 5;  // staged streams per row (X, W or z_{i-2}, r, Kx, Ky)
 
 // Chebyshev coefficients of the fused passes live in constant memory (one slot per
 // context): uniform per-step scalars then cost LDC through the constant cache instead
@@ -81,10 +92,72 @@ __device__ __forceinline__ void st2m(double *p, double2 v, bool a, bool b) {
         if (b) p[1] = v.y;
     }
 }
+__device__ __forceinline__ void cp16(void *sdst, const double *gsrc) {
+    asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(
+                     (uint32_t)__cvta_generic_to_shared(sdst)),
+                 "l"(gsrc)
+                 : "memory");
+}
+__device__ __forceinline__ void cp_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
+template <int N>
+__device__ __forceinline__ void cp_wait() {
+    asm volatile("cp.async.wait_group %0;" ::"n"(N) : "memory");
+}
 __device__ __forceinline__ double wsum(double v) {
 #pragma unroll
     for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
     return v;
+}
+
+// Tensor-memory (TMEM) delay lines (TEA_TB_TMEM): each thread owns one TMEM lane (warp w of
+// the CTA reaches lanes 32(w%4)..32(w%4)+31) and keeps its Kx, Ky, r delay slots there --
+// 16 32-bit columns per slot (Kx double2 in 0-3, Ky in 4-7, r in 8-11), 8 slots = 128
+// columns per warp quarter. tcgen05.st / tcgen05.ld (.32x32b) run on the tensor-memory
+// datapath, not on the L1TEX pipe that the shared-memory rings and the shuffles share
+// (tools/tmem_probe.cu: ~165 B/clk/SM of TMEM reads vs ~110 of shared memory at 12 warps).
+__device__ __forceinline__ uint32_t d_lo(double v) { return (uint32_t)__double_as_longlong(v); }
+__device__ __forceinline__ uint32_t d_hi(double v) {
+    return (uint32_t)((unsigned long long)__double_as_longlong(v) >> 32);
+}
+__device__ __forceinline__ double d_of(uint32_t lo, uint32_t hi) {
+    return __longlong_as_double(((long long)hi << 32) | lo);
+}
+__device__ __forceinline__ void tm_st12(uint32_t a, double2 kx, double2 ky, double2 r) {
+    asm volatile(
+        "tcgen05.st.sync.aligned.32x32b.x8.b32 [%0], {%1, %2, %3, %4, %5, %6, %7, %8};\n\t"
+        "tcgen05.st.sync.aligned.32x32b.x4.b32 [%9], {%10, %11, %12, %13};" ::"r"(a),
+        "r"(d_lo(kx.x)), "r"(d_hi(kx.x)), "r"(d_lo(kx.y)), "r"(d_hi(kx.y)), "r"(d_lo(ky.x)),
+        "r"(d_hi(ky.x)), "r"(d_lo(ky.y)), "r"(d_hi(ky.y)), "r"(a + 8u), "r"(d_lo(r.x)),
+        "r"(d_hi(r.x)), "r"(d_lo(r.y)), "r"(d_hi(r.y))
+        : "memory");
+}
+struct TmRow {
+    uint32_t v[12];
+};
+__device__ __forceinline__ void tm_ld12(uint32_t a, TmRow &o) {
+    asm volatile(
+        "tcgen05.ld.sync.aligned.32x32b.x8.b32 {%0, %1, %2, %3, %4, %5, %6, %7}, [%12];\n\t"
+        "tcgen05.ld.sync.aligned.32x32b.x4.b32 {%8, %9, %10, %11}, [%13];"
+        : "=r"(o.v[0]), "=r"(o.v[1]), "=r"(o.v[2]), "=r"(o.v[3]), "=r"(o.v[4]), "=r"(o.v[5]),
+          "=r"(o.v[6]), "=r"(o.v[7]), "=r"(o.v[8]), "=r"(o.v[9]), "=r"(o.v[10]), "=r"(o.v[11])
+        : "r"(a), "r"(a + 8u)
+        : "memory");
+}
+// wait for every outstanding tcgen05.ld; the registers are in/out operands so no use of
+// them can be scheduled above the wait
+__device__ __forceinline__ void tm_wait_ld(TmRow &o) {
+    asm volatile("tcgen05.wait::ld.sync.aligned;"
+                 : "+r"(o.v[0]), "+r"(o.v[1]), "+r"(o.v[2]), "+r"(o.v[3]), "+r"(o.v[4]),
+                   "+r"(o.v[5]), "+r"(o.v[6]), "+r"(o.v[7]), "+r"(o.v[8]), "+r"(o.v[9]),
+                   "+r"(o.v[10]), "+r"(o.v[11])
+                 :
+                 : "memory");
+}
+__device__ __forceinline__ void tm_wait_st() {
+    asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
+}
+__device__ __forceinline__ double2 tm_get(const TmRow &o, int i) {
+    return make_double2(d_of(o.v[4 * i], o.v[4 * i + 1]), d_of(o.v[4 * i + 2], o.v[4 * i + 3]));
 }
 
 // Deterministic two-value grid reduction (same scheme as tea_kernels.cu).
@@ -157,7 +230,14 @@ constexpr int kTbUnroll = TEA_TB_UNROLL;  // measured: 2 (step t+1 of row k over
 
 // dynamic shared memory of a pass: the Kx, Ky, r delay rings (depth 8, one double2 per
 // thread and row)
-constexpr size_t tb_smem_bytes() { return sizeof(double2) * 3 * 8 * kTbT; }
+// (TEA_TB_TMEM: the rings live in TMEM; the request then holds the cp.async row staging
+// and caps residency at 4 CTAs per SM so 4 x kTmCols TMEM columns always fit)
+constexpr size_t tb_smem_bytes() {
+    return TEA_TB_CPA > 0 ? (sizeof(double2) * kTbNS * (TEA_TB_CPA + 1) * kTbT > 48u * 1024u
+                                 ? sizeof(double2) * kTbNS * (TEA_TB_CPA + 1) * kTbT
+                                 : 48u * 1024u)
+                          : sizeof(double2) * 3 * 8 * kTbT;
+}
 
 template <int M>
 struct TbGeom {
@@ -181,6 +261,10 @@ struct TbGeom {
                        // slower: profiles/r01_tb_variants2.txt)
 #endif
 #define TB_REG_R (TEA_TB_REGLINES >= 1)
+#if TEA_TB_TMEM && TEA_TB_REGLINES
+#error "TEA_TB_TMEM replaces the delay lines; TEA_TB_REGLINES must be 0"
+#endif
+constexpr int kTmCols = 128;  // TMEM columns per CTA: 8 slots x 16 per warp quarter
 template <int M, bool FIRST, bool FUSE, bool LAST>
 __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     k_cheb_tb(const double *__restrict__ rin, const double *__restrict__ win,
@@ -219,12 +303,38 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         }
     }
     const double2 z0 = make_double2(0.0, 0.0);
+#if TEA_TB_TMEM
+    static_assert(kTbW % 4 == 0 || kTbW < 4, "warp quarters");
+    (void)ringKx;
+    (void)ringKy;
+    (void)ringR;
+    // one warp allocates the CTA's TMEM columns; every warp then owns lanes 32(w%4).. and
+    // a 128-column group per 4 warps. The dynamic shared memory request (tb_smem_bytes)
+    // keeps at most 4 CTAs per SM, so 4 x kTmCols <= 512 columns always fit.
+    __shared__ uint32_t tm_base_sh;
+    constexpr int kTmAlloc = kTmCols * ((kTbW + 3) / 4);
+    static_assert(kTmAlloc == 128 || kTmAlloc == 256, "TMEM allocation: power of two");
+    if ((threadIdx.x >> 5) == 0) {
+        asm volatile("tcgen05.alloc.cta_group::1.sync.aligned.shared::cta.b32 [%0], %1;" ::"r"(
+                         (uint32_t)__cvta_generic_to_shared(&tm_base_sh)),
+                     "n"(kTmAlloc)
+                     : "memory");
+        asm volatile("tcgen05.relinquish_alloc_permit.cta_group::1.sync.aligned;" ::: "memory");
+    }
+    asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory");
+    __syncthreads();
+    asm volatile("tcgen05.fence::after_thread_sync;" ::: "memory");
+    const uint32_t tm = tm_base_sh + ((uint32_t)(((threadIdx.x >> 5) & 3) * 32) << 16) +
+                        (uint32_t)(((threadIdx.x >> 5) >> 2) * kTmCols);
+    for (int d = 0; d < D; ++d) tm_st12(tm + 16u * d, z0, z0, z0);
+#else
     for (int d = 0; d < D; ++d) {
         ringKx[d][threadIdx.x] = z0;
         ringKy[d][threadIdx.x] = z0;
         ringR[d][threadIdx.x] = z0;
     }
     __syncthreads();
+#endif
 
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5, tid = threadIdx.x;
     (void)tid;
@@ -266,7 +376,43 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         pKx = ldg2c(Kx + o);
         pKy = ldg2c(Ky + o);
     };
+#if TB_CPA
+    // input rows staged TEA_TB_CPA rows ahead by cp.async into per-thread shared-memory slots
+    // (each thread copies and later reads back only its own 16 B per stream, so no
+    // barriers; slots the thread never fills stay zero). More bytes in flight per warp
+    // than one prefetched register row: the one-row version stalled on the load of the
+    // next row (ncu: 41% of stall samples on the first use of the prefetched row).
+    constexpr int P = TEA_TB_CPA, NSL = P + 1;
+    double2(*cpa)[kTbNS][kTbT] = reinterpret_cast<double2(*)[kTbNS][kTbT]>(tb_smem);
+    for (int sl = 0; sl < NSL; ++sl)
+#pragma unroll
+        for (int q = 0; q < kTbNS; ++q) cpa[sl][q][threadIdx.x] = z0;
+    auto issue = [&](long long o, int sl) {
+        if (ld_ok) {
+            if (FIRST) {
+                cp16(&cpa[sl][0][threadIdx.x], rin + o);
+                if (FUSE) cp16(&cpa[sl][1][threadIdx.x], win + o);
+            } else {
+                cp16(&cpa[sl][0][threadIdx.x], zin1 + o);
+                cp16(&cpa[sl][1][threadIdx.x], zin2 + o);
+                cp16(&cpa[sl][2][threadIdx.x], rin + o);
+            }
+            cp16(&cpa[sl][3][threadIdx.x], Kx + o);
+            cp16(&cpa[sl][4][threadIdx.x], Ky + o);
+        }
+        cp_commit();  // one group per row, empty or not, so wait_group counts rows
+    };
+#pragma unroll
+    for (int i = 0; i < P; ++i) {
+        if (kt0 < kt1 && kbeg + i < kend)
+            issue(orow + (long long)i * pitch, i);
+        else
+            cp_commit();
+    }
+    int cs = 0;  // slot of row k
+#else
     if (kt0 < kt1) load(orow);
+#endif
 #if TEA_TB_L2PF
     // L2 prefetch TEA_TB_L2PF rows ahead through the TMA unit (one lane, no registers, no
     // L1TEX wavefronts): the one-row register prefetch then hits L2
@@ -292,8 +438,30 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
 #endif
 #pragma unroll(kTbUnroll)
     for (int k = kbeg; k < kend; ++k, orow += pitch, head = (head + 1) & (D - 1)) {
+#if TB_CPA
+        cp_wait<P - 1>();  // row k's group (the oldest outstanding) has landed
+        const double2 X0 = cpa[cs][0][threadIdx.x];
+        const double2 KX = cpa[cs][3][threadIdx.x], KY = cpa[cs][4][threadIdx.x];
+        double2 X = X0, Wv = z0, Z2 = z0, RR = z0;
+        if (FIRST) {
+            if (FUSE) Wv = cpa[cs][1][threadIdx.x];
+        } else {
+            Z2 = cpa[cs][1][threadIdx.x];
+            RR = cpa[cs][2][threadIdx.x];
+        }
+        {
+            // row k+P goes into the slot row k-1 used (read a full iteration ago)
+            const int ns = cs == 0 ? P : cs - 1;
+            if (kt0 < kt1 && k + P < kend)
+                issue(orow + (long long)P * pitch, ns);
+            else
+                cp_commit();
+            cs = cs == P ? 0 : cs + 1;
+        }
+#else
         double2 X = pX, Wv = pW, Z2 = pZ2, KX = pKx, KY = pKy, RR = pR;
         if (k + 1 < kend) load(orow + pitch);
+#endif
 #if TEA_TB_L2PF
         if (lane == 0 && pfb > 0 && k + TEA_TB_L2PF < kend) {
             const long long o = orow + (long long)TEA_TB_L2PF * pitch;
@@ -319,7 +487,15 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         }
         // delay lines: shared-memory rings, or register shift registers (index i holds
         // row k - i; the step loop is unrolled, so step t's lag t is a compile-time index)
-#if TB_REG_K
+#if TEA_TB_TMEM
+        // the previous row's store must land before this row's loads read it back
+        tm_wait_st();
+        tm_st12(tm + 16u * head, KX, KY, rk);
+        TmRow tmA;
+        tm_ld12(tm + 16u * ((head - 1) & (D - 1)), tmA);
+        tm_wait_ld(tmA);
+        double2 ky_up = KY;  // Ky of row q+1 for step 1: this row's
+#elif TB_REG_K
 #pragma unroll
         for (int i = M; i > 0; --i) {
             rKx[i] = rKx[i - 1];
@@ -331,7 +507,8 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         ringKx[head][tid] = KX;
         ringKy[head][tid] = KY;
 #endif
-#if TB_REG_R
+#if TEA_TB_TMEM
+#elif TB_REG_R
 #pragma unroll
         for (int i = M; i > 0; --i) rR[i] = rR[i - 1];
         rR[0] = rk;
@@ -347,14 +524,22 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         for (int t = 1; t <= M; ++t) {
             const int q = k - t;
             const int sq = (head - t) & (D - 1), sq1 = (head - t + 1) & (D - 1);
-#if TB_REG_K
+#if TEA_TB_TMEM
+            // slot of row q = k - t is in tmA; issue the next step's slot before computing
+            const double2 kx = tm_get(tmA, 0), kyc = tm_get(tmA, 1), rq = tm_get(tmA, 2);
+            const double2 kyn = ky_up;
+            ky_up = kyc;
+            TmRow tmB;
+            if (t < M) tm_ld12(tm + 16u * ((head - t - 1) & (D - 1)), tmB);
+#elif TB_REG_K
             const double2 kx = rKx[t], kyc = rKy[t], kyn = rKy[t - 1];
 #else
             const double2 kx = ringKx[sq][tid];
             const double2 kyc = ringKy[sq][tid];
             const double2 kyn = ringKy[sq1][tid];
 #endif
-#if TB_REG_R
+#if TEA_TB_TMEM
+#elif TB_REG_R
             const double2 rq = rR[t];
 #else
             const double2 rq = ringR[sq][tid];
@@ -413,8 +598,22 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                     }
                 }
             }
+#if TEA_TB_TMEM
+            if (t < M) {
+                tm_wait_ld(tmB);
+                tmA = tmB;
+            }
+#endif
         }
     }
+#if TEA_TB_TMEM
+    asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory");
+    __syncthreads();
+    if ((threadIdx.x >> 5) == 0)
+        asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tm_base_sh),
+                     "n"(kTmAlloc)
+                     : "memory");
+#endif
     if (LAST) {
         double t0, t1;
         if (grid_reduce2(dot0, dot1, a.partials, &S->ticket, &t0, &t1)) {
