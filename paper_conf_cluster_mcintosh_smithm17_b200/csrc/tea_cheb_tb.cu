@@ -227,6 +227,17 @@ __device__ bool grid_arrive2(unsigned *ticket) {
 #endif
 constexpr int kTbUnroll = TEA_TB_UNROLL;  // measured: 2 (step t+1 of row k overlapping
                                           // step t of row k+1) costs registers, no gain
+#ifndef TEA_TB_UNROLL_L
+#define TEA_TB_UNROLL_L 3
+#endif
+#ifndef TEA_TB_CPA_L
+#define TEA_TB_CPA_L 2
+#endif
+// row-loop unroll and cp.async depth of the non-first passes (measured separately:
+// profiles/r01g_tmem_cpa.txt; the first pass carries r, w and more registers)
+constexpr int kTbUnrollL = TEA_TB_UNROLL_L;
+constexpr int kTbCpaL = TEA_TB_CPA > 0 ? TEA_TB_CPA_L : 0;
+static_assert(TEA_TB_CPA == 0 || (TEA_TB_CPA_L >= 1 && TEA_TB_CPA_L <= TEA_TB_CPA), "staging depth");
 
 // dynamic shared memory of a pass: the Kx, Ky, r delay rings (depth 8, one double2 per
 // thread and row)
@@ -382,7 +393,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     // barriers; slots the thread never fills stay zero). More bytes in flight per warp
     // than one prefetched register row: the one-row version stalled on the load of the
     // next row (ncu: 41% of stall samples on the first use of the prefetched row).
-    constexpr int P = TEA_TB_CPA, NSL = P + 1;
+    constexpr int P = FIRST ? TEA_TB_CPA : kTbCpaL, NSL = P + 1;
     double2(*cpa)[kTbNS][kTbT] = reinterpret_cast<double2(*)[kTbNS][kTbT]>(tb_smem);
     for (int sl = 0; sl < NSL; ++sl)
 #pragma unroll
@@ -436,7 +447,10 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
 #pragma unroll
     for (int i = 0; i <= M; ++i) rR[i] = z0;
 #endif
-#pragma unroll(kTbUnroll)
+    // the later passes (fewer live registers) unroll the row loop by the window period 3:
+    // the W[t][*] rotation becomes register renaming instead of ~50 moves per row
+    constexpr int UNR = FIRST ? kTbUnroll : kTbUnrollL;
+#pragma unroll(UNR)
     for (int k = kbeg; k < kend; ++k, orow += pitch, head = (head + 1) & (D - 1)) {
 #if TB_CPA
         cp_wait<P - 1>();  // row k's group (the oldest outstanding) has landed
