@@ -14,13 +14,14 @@
 // computes z_t at row k - t for t = 1..M. Each step keeps its last three rows in
 // registers (the stencil window of the next step; its oldest row is also the z_{t-2}
 // pointwise term of step t+2); x-neighbours come from warp shuffles. The pointwise
-// operands Kx, Ky, r (and z_{i-2}) are needed M rows after they are loaded: they wait in
-// per-thread shared-memory delay lines (each thread reads back only what it wrote, so no
-// barriers). Every step loses one valid column per side (no edge loads): strips overlap
-// and each produces 64 - 2*ceil_even(M) output columns. A CTA tile of ty output rows
-// runs ty + 2M row-iterations (pipeline fill/drain).
-//
-// Single-block only (no extended bounds); blocks with neighbours use the per-step kernels.
+// operands Kx, Ky, r and the diagonal of A are needed up to M rows after they are loaded:
+// they wait in a per-thread ring of row slots in tensor memory (TMEM, tcgen05.st/ld), off
+// the L1TEX pipe the shuffles use. Input rows arrive by cp.async into per-thread
+// shared-memory slots P rows ahead of the march (bytes in flight). Every step loses one
+// valid column per side (no edge loads): strips overlap and each produces
+// 64 - 2*ceil_even(M) output columns. A CTA tile of ty output rows runs ty + 2M
+// row-iterations (pipeline fill/drain). The region R may include extended bounds toward
+// neighbour blocks (matrix powers across blocks).
 #include "tea_internal.h"
 
 #include <mutex>
@@ -35,15 +36,8 @@ namespace tea {
 // but only 3 CTAs of 4 warps.
 constexpr int kTbW = TEA_TB_WARPS;
 constexpr int kTbT = 32 * kTbW;
-#ifndef TEA_TB_TMEM
-#define TEA_TB_TMEM 1  // Kx, Ky, r delay lines in tensor memory (see tm_st12)
-#endif
 #ifndef TEA_TB_CPA
-#define TEA_TB_CPA 4  // rows of cp.async input staging ahead of the march (0: one register row)
-#endif
-#define TB_CPA (TEA_TB_CPA > 0)
-#if TB_CPA && !TEA_TB_TMEM
-#error "TEA_TB_CPA stages rows in the shared memory the rings would use: needs TEA_TB_TMEM"
+#define TEA_TB_CPA 4  // rows of cp.async input staging ahead of the march (first pass)
 #endif
 constexpr int kTbNS = 5;  // staged streams per row (X, W or z_{i-2}, r, Kx, Ky)
 
@@ -81,9 +75,6 @@ cudaError_t tb_coef_upload(int slot, const Scalars *S, cudaStream_t st) {
 
 namespace {
 
-__device__ __forceinline__ double2 ldg2c(const double *p) {
-    return __ldg(reinterpret_cast<const double2 *>(p));
-}
 __device__ __forceinline__ void st2m(double *p, double2 v, bool a, bool b) {
     if (a && b) {
         *reinterpret_cast<double2 *>(p) = v;
@@ -109,10 +100,10 @@ __device__ __forceinline__ double wsum(double v) {
     return v;
 }
 
-// Tensor-memory (TMEM) delay lines (TEA_TB_TMEM): each thread owns one TMEM lane (warp w of
-// the CTA reaches lanes 32(w%4)..32(w%4)+31) and keeps its Kx, Ky, r delay slots there --
-// 16 32-bit columns per slot (Kx double2 in 0-3, Ky in 4-7, r in 8-11), 8 slots = 128
-// columns per warp quarter. tcgen05.st / tcgen05.ld (.32x32b) run on the tensor-memory
+// Tensor-memory (TMEM) delay lines: each thread owns one TMEM lane (warp w of
+// the CTA reaches lanes 32(w%4)..32(w%4)+31) and keeps its row slots there -- 16 32-bit
+// columns per slot (Kx double2 in 0-3, Ky in 4-7, r in 8-11, diag(A) in 12-15), 8 slots =
+// 128 columns per warp quarter. tcgen05.st / tcgen05.ld (.32x32b) run on the tensor-memory
 // datapath, not on the L1TEX pipe that the shared-memory rings and the shuffles share
 // (tools/tmem_probe.cu: ~165 B/clk/SM of TMEM reads vs ~110 of shared memory at 12 warps).
 __device__ __forceinline__ uint32_t d_lo(double v) { return (uint32_t)__double_as_longlong(v); }
@@ -122,18 +113,44 @@ __device__ __forceinline__ uint32_t d_hi(double v) {
 __device__ __forceinline__ double d_of(uint32_t lo, uint32_t hi) {
     return __longlong_as_double(((long long)hi << 32) | lo);
 }
-__device__ __forceinline__ void tm_st12(uint32_t a, double2 kx, double2 ky, double2 r) {
+__device__ __forceinline__ void tm_st16(uint32_t a, double2 v0, double2 v1, double2 v2,
+                                        double2 v3) {
+    asm volatile(
+        "tcgen05.st.sync.aligned.32x32b.x16.b32 [%0], {%1, %2, %3, %4, %5, %6, %7, %8, %9, "
+        "%10, %11, %12, %13, %14, %15, %16};" ::"r"(a),
+        "r"(d_lo(v0.x)), "r"(d_hi(v0.x)), "r"(d_lo(v0.y)), "r"(d_hi(v0.y)), "r"(d_lo(v1.x)),
+        "r"(d_hi(v1.x)), "r"(d_lo(v1.y)), "r"(d_hi(v1.y)), "r"(d_lo(v2.x)), "r"(d_hi(v2.x)),
+        "r"(d_lo(v2.y)), "r"(d_hi(v2.y)), "r"(d_lo(v3.x)), "r"(d_hi(v3.x)), "r"(d_lo(v3.y)),
+        "r"(d_hi(v3.y))
+        : "memory");
+}
+__device__ __forceinline__ void tm_st12(uint32_t a, double2 v0, double2 v1, double2 v2) {
     asm volatile(
         "tcgen05.st.sync.aligned.32x32b.x8.b32 [%0], {%1, %2, %3, %4, %5, %6, %7, %8};\n\t"
         "tcgen05.st.sync.aligned.32x32b.x4.b32 [%9], {%10, %11, %12, %13};" ::"r"(a),
-        "r"(d_lo(kx.x)), "r"(d_hi(kx.x)), "r"(d_lo(kx.y)), "r"(d_hi(kx.y)), "r"(d_lo(ky.x)),
-        "r"(d_hi(ky.x)), "r"(d_lo(ky.y)), "r"(d_hi(ky.y)), "r"(a + 8u), "r"(d_lo(r.x)),
-        "r"(d_hi(r.x)), "r"(d_lo(r.y)), "r"(d_hi(r.y))
+        "r"(d_lo(v0.x)), "r"(d_hi(v0.x)), "r"(d_lo(v0.y)), "r"(d_hi(v0.y)), "r"(d_lo(v1.x)),
+        "r"(d_hi(v1.x)), "r"(d_lo(v1.y)), "r"(d_hi(v1.y)), "r"(a + 8u), "r"(d_lo(v2.x)),
+        "r"(d_hi(v2.x)), "r"(d_lo(v2.y)), "r"(d_hi(v2.y))
         : "memory");
 }
+__device__ __forceinline__ void tm_st4(uint32_t a, double2 v) {
+    asm volatile("tcgen05.st.sync.aligned.32x32b.x4.b32 [%0], {%1, %2, %3, %4};" ::"r"(a),
+                 "r"(d_lo(v.x)), "r"(d_hi(v.x)), "r"(d_lo(v.y)), "r"(d_hi(v.y))
+                 : "memory");
+}
 struct TmRow {
-    uint32_t v[12];
+    uint32_t v[16];
 };
+__device__ __forceinline__ void tm_ld16(uint32_t a, TmRow &o) {
+    asm volatile(
+        "tcgen05.ld.sync.aligned.32x32b.x16.b32 {%0, %1, %2, %3, %4, %5, %6, %7, %8, %9, %10, "
+        "%11, %12, %13, %14, %15}, [%16];"
+        : "=r"(o.v[0]), "=r"(o.v[1]), "=r"(o.v[2]), "=r"(o.v[3]), "=r"(o.v[4]), "=r"(o.v[5]),
+          "=r"(o.v[6]), "=r"(o.v[7]), "=r"(o.v[8]), "=r"(o.v[9]), "=r"(o.v[10]), "=r"(o.v[11]),
+          "=r"(o.v[12]), "=r"(o.v[13]), "=r"(o.v[14]), "=r"(o.v[15])
+        : "r"(a)
+        : "memory");
+}
 __device__ __forceinline__ void tm_ld12(uint32_t a, TmRow &o) {
     asm volatile(
         "tcgen05.ld.sync.aligned.32x32b.x8.b32 {%0, %1, %2, %3, %4, %5, %6, %7}, [%12];\n\t"
@@ -149,7 +166,8 @@ __device__ __forceinline__ void tm_wait_ld(TmRow &o) {
     asm volatile("tcgen05.wait::ld.sync.aligned;"
                  : "+r"(o.v[0]), "+r"(o.v[1]), "+r"(o.v[2]), "+r"(o.v[3]), "+r"(o.v[4]),
                    "+r"(o.v[5]), "+r"(o.v[6]), "+r"(o.v[7]), "+r"(o.v[8]), "+r"(o.v[9]),
-                   "+r"(o.v[10]), "+r"(o.v[11])
+                   "+r"(o.v[10]), "+r"(o.v[11]), "+r"(o.v[12]), "+r"(o.v[13]), "+r"(o.v[14]),
+                   "+r"(o.v[15])
                  :
                  : "memory");
 }
@@ -223,59 +241,46 @@ __device__ bool grid_arrive2(unsigned *ticket) {
 }  // namespace
 
 #ifndef TEA_TB_UNROLL
-#define TEA_TB_UNROLL 1
+#define TEA_TB_UNROLL 3
 #endif
-constexpr int kTbUnroll = TEA_TB_UNROLL;  // measured: 2 (step t+1 of row k overlapping
-                                          // step t of row k+1) costs registers, no gain
 #ifndef TEA_TB_UNROLL_L
 #define TEA_TB_UNROLL_L 3
 #endif
 #ifndef TEA_TB_CPA_L
 #define TEA_TB_CPA_L 2
 #endif
-// row-loop unroll and cp.async depth of the non-first passes (measured separately:
-// profiles/r01g_tmem_cpa.txt; the first pass carries r, w and more registers)
-constexpr int kTbUnrollL = TEA_TB_UNROLL_L;
-constexpr int kTbCpaL = TEA_TB_CPA > 0 ? TEA_TB_CPA_L : 0;
-static_assert(TEA_TB_CPA == 0 || (TEA_TB_CPA_L >= 1 && TEA_TB_CPA_L <= TEA_TB_CPA), "staging depth");
+#ifndef TEA_TB_DIAG
+#define TEA_TB_DIAG 1
+#endif
+// Row-loop unroll and cp.async depth of the first pass (carries r, w and the update) and of
+// the later passes, measured separately (profiles/r01g_tmem_cpa.txt): unrolling by the
+// window period 3 turns the W[t][*] rotation into register renaming instead of ~50 moves per
+// row; with 3 CTAs per SM requested (TEA_TB_MINB) the first pass still fits 152 registers.
+constexpr int kTbUnroll = TEA_TB_UNROLL, kTbUnrollL = TEA_TB_UNROLL_L;
+constexpr int kTbCpa = TEA_TB_CPA, kTbCpaL = TEA_TB_CPA_L;
+static_assert(kTbCpa >= 1 && kTbCpaL >= 1 && kTbCpaL <= kTbCpa, "staging depth");
 
-// dynamic shared memory of a pass: the Kx, Ky, r delay rings (depth 8, one double2 per
-// thread and row)
-// (TEA_TB_TMEM: the rings live in TMEM; the request then holds the cp.async row staging
-// and caps residency at 4 CTAs per SM so 4 x kTmCols TMEM columns always fit)
+// dynamic shared memory of a pass: the cp.async row staging; at least 48 KB so at most 4
+// CTAs are resident per SM and 4 x kTmCols TMEM columns always fit in the SM's 512
 constexpr size_t tb_smem_bytes() {
-    return TEA_TB_CPA > 0 ? (sizeof(double2) * kTbNS * (TEA_TB_CPA + 1) * kTbT > 48u * 1024u
-                                 ? sizeof(double2) * kTbNS * (TEA_TB_CPA + 1) * kTbT
-                                 : 48u * 1024u)
-                          : sizeof(double2) * 3 * 8 * kTbT;
+    return sizeof(double2) * kTbNS * (kTbCpa + 1) * kTbT > 48u * 1024u
+               ? sizeof(double2) * kTbNS * (kTbCpa + 1) * kTbT
+               : 48u * 1024u;
 }
 
 template <int M>
 struct TbGeom {
     static constexpr int MR = (M + 1) & ~1;  // margin, even (double2 alignment)
     static constexpr int OW = kStrip - 2 * MR;  // output columns per warp strip
-    static constexpr int D = 8;  // delay-line depth (rows k-M-1..k fit for M <= 6); a power of
-                                 // two so slots are (head - t) & 7, not a division
+    static constexpr int D = 8;  // TMEM ring depth (rows k-M-1..k fit for M <= 6); a power of
+                                 // two so slots are (head - t) & 7
 };
 
 #ifndef TEA_TB_MINB
-#define TEA_TB_MINB 1
+#define TEA_TB_MINB 3
 #endif
-#ifndef TEA_TB_REGLINES
-#define TEA_TB_REGLINES 0  // 1: Kx, Ky and r lines in registers (measured slower: 225 regs,
-                            // 2 CTAs/SM, 737 vs 660 us/outer, profiles/r01_tb_reglines.txt);
-                            // 2: r only
-#endif
-#define TB_REG_K (TEA_TB_REGLINES == 1)
-#ifndef TEA_TB_L2PF
-#define TEA_TB_L2PF 0  // rows of L2 bulk-prefetch distance (0 = off; 3, 6, 10 measured
-                       // slower: profiles/r01_tb_variants2.txt)
-#endif
-#define TB_REG_R (TEA_TB_REGLINES >= 1)
-#if TEA_TB_TMEM && TEA_TB_REGLINES
-#error "TEA_TB_TMEM replaces the delay lines; TEA_TB_REGLINES must be 0"
-#endif
-constexpr int kTmCols = 128;  // TMEM columns per CTA: 8 slots x 16 per warp quarter
+constexpr int kTmCols = 128;  // TMEM columns per 4 warps: 8 slots x 16 per warp quarter
+
 template <int M, bool FIRST, bool FUSE, bool LAST>
 __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     k_cheb_tb(const double *__restrict__ rin, const double *__restrict__ win,
@@ -286,11 +291,9 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
               int step0, int restart) {
     using G = TbGeom<M>;
     constexpr int D = G::D;
-    static_assert(M <= 6, "delay lines hold M+2 rows");
+    static_assert(M <= 6, "the TMEM ring holds M+2 rows");
+    static_assert(kTbW <= 4 || kTbW % 4 == 0, "warp quarters");
     extern __shared__ double2 tb_smem[];
-    double2(*ringKx)[kTbT] = reinterpret_cast<double2(*)[kTbT]>(tb_smem);
-    double2(*ringKy)[kTbT] = ringKx + D;
-    double2(*ringR)[kTbT] = ringKy + D;
     const double(*coef)[kMaxS] = c_tb_coef[a.coef_slot];
 
     Scalars *S = a.S;
@@ -314,14 +317,8 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         }
     }
     const double2 z0 = make_double2(0.0, 0.0);
-#if TEA_TB_TMEM
-    static_assert(kTbW % 4 == 0 || kTbW < 4, "warp quarters");
-    (void)ringKx;
-    (void)ringKy;
-    (void)ringR;
-    // one warp allocates the CTA's TMEM columns; every warp then owns lanes 32(w%4).. and
-    // a 128-column group per 4 warps. The dynamic shared memory request (tb_smem_bytes)
-    // keeps at most 4 CTAs per SM, so 4 x kTmCols <= 512 columns always fit.
+    // One warp allocates the CTA's TMEM columns; warp w then owns lanes 32(w%4).. and a
+    // 128-column group per 4 warps: per thread a private ring of D row slots (tm_st16).
     __shared__ uint32_t tm_base_sh;
     constexpr int kTmAlloc = kTmCols * ((kTbW + 3) / 4);
     static_assert(kTmAlloc == 128 || kTmAlloc == 256, "TMEM allocation: power of two");
@@ -337,18 +334,9 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     asm volatile("tcgen05.fence::after_thread_sync;" ::: "memory");
     const uint32_t tm = tm_base_sh + ((uint32_t)(((threadIdx.x >> 5) & 3) * 32) << 16) +
                         (uint32_t)(((threadIdx.x >> 5) >> 2) * kTmCols);
-    for (int d = 0; d < D; ++d) tm_st12(tm + 16u * d, z0, z0, z0);
-#else
-    for (int d = 0; d < D; ++d) {
-        ringKx[d][threadIdx.x] = z0;
-        ringKy[d][threadIdx.x] = z0;
-        ringR[d][threadIdx.x] = z0;
-    }
-    __syncthreads();
-#endif
+    for (int d = 0; d < D; ++d) tm_st16(tm + 16u * d, z0, z0, z0, z0);  // zero ring
 
-    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5, tid = threadIdx.x;
-    (void)tid;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const int strip = blockIdx.x * kTbW + warp;
     // strips tile the output region R (which may reach into the halo on sides with a
     // neighbour block: extended bounds); first strip starts MR before it
@@ -370,30 +358,14 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     for (int t = 0; t < M; ++t) W[t][0] = W[t][1] = W[t][2] = z0;
     double dot0 = 0.0, dot1 = 0.0;
 
-    // prefetch registers for input row k; running element offsets (no k*pitch products)
-    double2 pX = z0, pW = z0, pZ2 = z0, pKx = z0, pKy = z0, pR = z0;
     const int kbeg = kt0 - M, kend = kt1 + M;
-    long long orow = (long long)kbeg * pitch + jA;  // offset of (jA, k)
-    auto load = [&](long long o) {
-        if (!ld_ok) return;
-        if (FIRST) {
-            pX = ldg2c(rin + o);
-            if (FUSE) pW = ldg2c(win + o);
-        } else {
-            pX = ldg2c(zin1 + o);
-            pZ2 = ldg2c(zin2 + o);
-            pR = ldg2c(rin + o);
-        }
-        pKx = ldg2c(Kx + o);
-        pKy = ldg2c(Ky + o);
-    };
-#if TB_CPA
-    // input rows staged TEA_TB_CPA rows ahead by cp.async into per-thread shared-memory slots
+    long long orow = (long long)kbeg * pitch + jA;  // offset of (jA, k); running, no k*pitch
+    // Input rows are staged P rows ahead by cp.async into per-thread shared-memory slots
     // (each thread copies and later reads back only its own 16 B per stream, so no
-    // barriers; slots the thread never fills stay zero). More bytes in flight per warp
-    // than one prefetched register row: the one-row version stalled on the load of the
-    // next row (ncu: 41% of stall samples on the first use of the prefetched row).
-    constexpr int P = FIRST ? TEA_TB_CPA : kTbCpaL, NSL = P + 1;
+    // barriers; slots the thread never fills stay zero): P rows of bytes in flight per
+    // warp. With one register-prefetched row the pass stalled on the load of the next row
+    // (ncu: 41% of stall samples on its first use; profiles/r01g_tmem_cpa.txt).
+    constexpr int P = FIRST ? kTbCpa : kTbCpaL, NSL = P + 1;
     double2(*cpa)[kTbNS][kTbT] = reinterpret_cast<double2(*)[kTbNS][kTbT]>(tb_smem);
     for (int sl = 0; sl < NSL; ++sl)
 #pragma unroll
@@ -420,43 +392,16 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         else
             cp_commit();
     }
-    int cs = 0;  // slot of row k
-#else
-    if (kt0 < kt1) load(orow);
-#endif
-#if TEA_TB_L2PF
-    // L2 prefetch TEA_TB_L2PF rows ahead through the TMA unit (one lane, no registers, no
-    // L1TEX wavefronts): the one-row register prefetch then hits L2
-    const int jA0 = __shfl_sync(0xffffffffu, jA, 0);
-    int pfb = (jlim - jA0) * 8;
-    pfb = pfb > kStrip * 8 ? kStrip * 8 : (pfb & ~15);
-    auto l2pf = [&](const double *base, long long o) {
-        asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(base + o), "r"(pfb)
-                     : "memory");
-    };
-#endif
-    int head = 0;  // ring slot of row k
+    int cs = 0;    // staging slot of row k
+    int head = 0;  // TMEM ring slot of row k
     double2 z2prev = z0;  // z_{i-2} input of the previous row (a one-row register delay)
-#if TB_REG_K
-    double2 rKx[M + 1], rKy[M + 1];
-#pragma unroll
-    for (int i = 0; i <= M; ++i) rKx[i] = rKy[i] = z0;
-#endif
-#if TB_REG_R
-    double2 rR[M + 1];
-#pragma unroll
-    for (int i = 0; i <= M; ++i) rR[i] = z0;
-#endif
-    // the later passes (fewer live registers) unroll the row loop by the window period 3:
-    // the W[t][*] rotation becomes register renaming instead of ~50 moves per row
     constexpr int UNR = FIRST ? kTbUnroll : kTbUnrollL;
 #pragma unroll(UNR)
     for (int k = kbeg; k < kend; ++k, orow += pitch, head = (head + 1) & (D - 1)) {
-#if TB_CPA
         cp_wait<P - 1>();  // row k's group (the oldest outstanding) has landed
-        const double2 X0 = cpa[cs][0][threadIdx.x];
+        double2 X = cpa[cs][0][threadIdx.x];
         const double2 KX = cpa[cs][3][threadIdx.x], KY = cpa[cs][4][threadIdx.x];
-        double2 X = X0, Wv = z0, Z2 = z0, RR = z0;
+        double2 Wv = z0, Z2 = z0, RR = z0;
         if (FIRST) {
             if (FUSE) Wv = cpa[cs][1][threadIdx.x];
         } else {
@@ -472,25 +417,6 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                 cp_commit();
             cs = cs == P ? 0 : cs + 1;
         }
-#else
-        double2 X = pX, Wv = pW, Z2 = pZ2, KX = pKx, KY = pKy, RR = pR;
-        if (k + 1 < kend) load(orow + pitch);
-#endif
-#if TEA_TB_L2PF
-        if (lane == 0 && pfb > 0 && k + TEA_TB_L2PF < kend) {
-            const long long o = orow + (long long)TEA_TB_L2PF * pitch;
-            if (FIRST) {
-                l2pf(rin, o);
-                if (FUSE) l2pf(win, o);
-            } else {
-                l2pf(zin1, o);
-                l2pf(zin2, o);
-                l2pf(rin, o);
-            }
-            l2pf(Kx, o);
-            l2pf(Ky, o);
-        }
-#endif
         double2 rk;
         if (FIRST) {
             if (FUSE) X = make_double2(X.x - alpha * Wv.x, X.y - alpha * Wv.y);
@@ -499,35 +425,26 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         } else {
             rk = RR;
         }
-        // delay lines: shared-memory rings, or register shift registers (index i holds
-        // row k - i; the step loop is unrolled, so step t's lag t is a compile-time index)
-#if TEA_TB_TMEM
-        // the previous row's store must land before this row's loads read it back
+        // step t works on row q = k - t and needs that row's Kx, Ky, r (and Ky of row q+1):
+        // they wait in this thread's TMEM ring. The previous row's store must land before
+        // this row's loads read it back.
         tm_wait_st();
         tm_st12(tm + 16u * head, KX, KY, rk);
         TmRow tmA;
-        tm_ld12(tm + 16u * ((head - 1) & (D - 1)), tmA);
+        tm_ld12(tm + 16u * ((head - 1) & (D - 1)), tmA);  // row k-1: step 1's operands
         tm_wait_ld(tmA);
-        double2 ky_up = KY;  // Ky of row q+1 for step 1: this row's
-#elif TB_REG_K
-#pragma unroll
-        for (int i = M; i > 0; --i) {
-            rKx[i] = rKx[i - 1];
-            rKy[i] = rKy[i - 1];
-        }
-        rKx[0] = KX;
-        rKy[0] = KY;
-#else
-        ringKx[head][tid] = KX;
-        ringKy[head][tid] = KY;
-#endif
-#if TEA_TB_TMEM
-#elif TB_REG_R
-#pragma unroll
-        for (int i = M; i > 0; --i) rR[i] = rR[i - 1];
-        rR[0] = rk;
-#else
-        ringR[head][tid] = rk;
+        double2 s_kx = tm_get(tmA, 0), s_ky = tm_get(tmA, 1), s_r = tm_get(tmA, 2), kyn = KY;
+#if TEA_TB_DIAG
+        // Row k-1 is completed now that its top faces (row k's Ky) are known: the diagonal
+        // of A (Listing 1: 1 + the sum of the cell's four face coefficients) is formed once
+        // per row here, not once per step, and joins the row's slot (columns 12-15).
+        // Kx(jA+2) (the face east of cell B) is the east lane's Kx(jA): one shuffle per row
+        // (lane 31's value only feeds the margin).
+        const double kxE = __shfl_down_sync(0xffffffffu, s_kx.x, 1);
+        double2 s_d;
+        s_d.x = 1.0 + (s_kx.x + s_kx.y) + (s_ky.x + KY.x);
+        s_d.y = 1.0 + (s_kx.y + kxE) + (s_ky.y + KY.y);
+        tm_st4(tm + 16u * ((head - 1) & (D - 1)) + 12u, s_d);
 #endif
         const double2 z2row = z2prev;  // z_{i-2} of row k-1
         if (!FIRST) z2prev = Z2;
@@ -537,29 +454,14 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
 #pragma unroll
         for (int t = 1; t <= M; ++t) {
             const int q = k - t;
-            const int sq = (head - t) & (D - 1), sq1 = (head - t + 1) & (D - 1);
-#if TEA_TB_TMEM
-            // slot of row q = k - t is in tmA; issue the next step's slot before computing
-            const double2 kx = tm_get(tmA, 0), kyc = tm_get(tmA, 1), rq = tm_get(tmA, 2);
-            const double2 kyn = ky_up;
-            ky_up = kyc;
+            // issue the next step's slot (row q-1) before computing this one
             TmRow tmB;
+#if TEA_TB_DIAG
+            if (t < M) tm_ld16(tm + 16u * ((head - t - 1) & (D - 1)), tmB);
+#else
             if (t < M) tm_ld12(tm + 16u * ((head - t - 1) & (D - 1)), tmB);
-#elif TB_REG_K
-            const double2 kx = rKx[t], kyc = rKy[t], kyn = rKy[t - 1];
-#else
-            const double2 kx = ringKx[sq][tid];
-            const double2 kyc = ringKy[sq][tid];
-            const double2 kyn = ringKy[sq1][tid];
 #endif
-#if TEA_TB_TMEM
-#elif TB_REG_R
-            const double2 rq = rR[t];
-#else
-            const double2 rq = ringR[sq][tid];
-#endif
-            (void)sq;
-            (void)sq1;
+            const double2 kx = s_kx, kyc = s_ky, rq = s_r;
             double2 z2;
             if (t == 1) {
                 z2 = FIRST ? z0 : z2row;
@@ -567,29 +469,52 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                 z2 = W[t >= 2 ? t - 2 : 0][0];
             }
             const double2 xm = W[t - 1][0], xc = W[t - 1][1], xp = W[t - 1][2];
+            const int ci = step0 - 2 + t;
+            const double cx = coef[0][ci], cz = coef[1][ci], cr = coef[2][ci], ca = coef[3][ci];
             // lane 0's left and lane 31's right neighbours are outside the strip: the
             // shuffles return the lane's own (finite) value, which only pollutes the
-            // overlap columns every step already discards -- no selects needed
+            // overlap columns every step already discards -- no selects needed.
+            // Dependency order: xp (the "up" row) is the row step t-1 produced in THIS
+            // row-iteration; everything else is older. Form the rest first, fold xp in last.
+            double2 zn;
+#if TEA_TB_DIAG
+            // z = cx X + cz z2 + cr r - ca (d X - sum_f K_f X_f)              (Listing 1)
+            // West neighbour of cell A from the west lane; the east term of cell B,
+            // Kx(jA+2) X(jA+2), is the east lane's own Kx(jA) X(jA) -- one product shuffled.
+            // The per-step coefficients only ever multiply vector registers (uniform
+            // operands, nothing hoisted into vector registers).
+            const double2 dg = s_d;
+            const double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
+            const double east = __shfl_down_sync(0xffffffffu, kx.x * xc.x, 1);
+            double2 base, nb;
+            base.x = cx * xc.x;
+            base.y = cx * xc.y;
+            if (!(FIRST && t == 1)) {
+                base.x = fma(cz, z2.x, base.x);
+                base.y = fma(cz, z2.y, base.y);
+            }
+            base.x = fma(cr, rq.x, base.x);
+            base.y = fma(cr, rq.y, base.y);
+            nb.x = fma(-dg.x, xc.x, fma(kx.x, left, fma(kx.y, xc.y, kyc.x * xm.x)));
+            nb.y = fma(-dg.y, xc.y, fma(kx.y, xc.x, fma(kyc.y, xm.y, east)));
+            zn.x = fma(ca, fma(kyn.x, xp.x, nb.x), base.x);
+            zn.y = fma(ca, fma(kyn.y, xp.y, nb.y), base.y);
+#else
             // x direction in flux form: A x = x + sum_faces K_f (x_c - x_f) (Listing 1
             // regrouped). gw = Kx_w (x_A - x_left) is formed by the lane that owns the face's
-            // Kx; its east neighbour receives it as -(its east flux). Two shuffles of x and
-            // one of the flux -- no shuffle of Kx.
+            // Kx; its east neighbour receives it as -(its east flux).
             const double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
             const double gw = kx.x * (xc.x - left);
             const double gm = kx.y * (xc.x - xc.y);
             const double ge = __shfl_down_sync(0xffffffffu, gw, 1);  // Kx_e (x_right - x_B)
-            // Dependency order: xp (the "up" row) is the row step t-1 produced in THIS
-            // row-iteration; everything else is older. Form the rest first, fold xp in last.
-            const int ci = step0 - 2 + t;
-            const double cx = coef[0][ci], cz = coef[1][ci], cr = coef[2][ci], ca = coef[3][ci];
             double2 AXo, base;  // A x without the up term; the step's x-independent part
             AXo.x = (1.0 + (kyn.x + kyc.x)) * xc.x - kyc.x * xm.x + (gw + gm);
             AXo.y = (1.0 + (kyn.y + kyc.y)) * xc.y - kyc.y * xm.y - (gm + ge);
             base.x = cx * xc.x + cz * z2.x + cr * rq.x;
             base.y = cx * xc.y + cz * z2.y + cr * rq.y;
-            double2 zn;
             zn.x = fma(-ca, fma(-kyn.x, xp.x, AXo.x), base.x);
             zn.y = fma(-ca, fma(-kyn.y, xp.y, AXo.y), base.y);
+#endif
             const bool rowout = q >= kt0 && q < kt1;
             if (t < M) {
                 const int tt = t < M ? t : M - 1;
@@ -612,22 +537,24 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                     }
                 }
             }
-#if TEA_TB_TMEM
             if (t < M) {
                 tm_wait_ld(tmB);
-                tmA = tmB;
-            }
+                kyn = kyc;  // Ky of row q = the top faces of row q-1
+                s_kx = tm_get(tmB, 0);
+                s_ky = tm_get(tmB, 1);
+                s_r = tm_get(tmB, 2);
+#if TEA_TB_DIAG
+                s_d = tm_get(tmB, 3);
 #endif
+            }
         }
     }
-#if TEA_TB_TMEM
     asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory");
     __syncthreads();
     if ((threadIdx.x >> 5) == 0)
         asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tm_base_sh),
                      "n"(kTmAlloc)
                      : "memory");
-#endif
     if (LAST) {
         double t0, t1;
         if (grid_reduce2(dot0, dot1, a.partials, &S->ticket, &t0, &t1)) {
