@@ -529,11 +529,11 @@ std::vector<int> tb_passes(int s, int mmax) {
 int tb_steps(const tea_ctx *c) {
     int m = c->opts.tb_steps;
     if (m == 0) {
-        // measured (profiles/r01_tb_sweep.txt): fusing pays once the working set
-        // (13 fields) leaves L2 -- 4096^2: 5 steps/pass 755 us vs 1520 us per outer;
-        // at 1024^2 (L2-resident) one kernel per step is faster (86 vs 87-100 us).
+        // measured (profiles/r01g_tmem_cpa.txt, TMEM/cp.async passes): 5 steps per pass
+        // beat one kernel per step from 640^2 up (50 vs 59 us per outer; 1024^2 72 vs 86,
+        // 4096^2 ~500 vs 1520); smaller CPPCG blocks run the persistent solver.
         const double cells = (double)c->blocks[0].L.bx * c->blocks[0].L.by;
-        m = cells >= 2.0e6 ? kTbMaxSteps : 1;
+        m = cells >= 4.0e5 ? kTbMaxSteps : 1;
     }
     return std::min(m, kTbMaxSteps);
 }
