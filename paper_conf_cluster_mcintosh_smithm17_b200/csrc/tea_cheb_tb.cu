@@ -497,6 +497,8 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             base.y = fma(cr, rq.y, base.y);
             nb.x = fma(-dg.x, xc.x, fma(kx.x, left, fma(kx.y, xc.y, kyc.x * xm.x)));
             nb.y = fma(-dg.y, xc.y, fma(kx.y, xc.x, fma(kyc.y, xm.y, east)));
+            // (folding ca into kyn to leave one dependent DFMA after xp costs a DMUL per cell
+            // and measured slower: profiles/r01g_tmem_cpa.txt)
             zn.x = fma(ca, fma(kyn.x, xp.x, nb.x), base.x);
             zn.y = fma(ca, fma(kyn.y, xp.y, nb.y), base.y);
 #else
