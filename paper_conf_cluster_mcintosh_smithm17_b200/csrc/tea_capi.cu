@@ -243,6 +243,14 @@ Launch plan_st(tea_ctx *c, const BlockCtx &b, const Region &R) {
     if (b.L.nz > 1) return plan_stencil3(R, b.L.nz, c->opts.tile_rows);
     return plan(c, R);
 }
+// the SpMV: large 2D blocks (where the default tile is the 32-row cap) get wave-fitted tiles
+Launch plan_spmv(tea_ctx *c, const BlockCtx &b, const Region &R) {
+    Launch L = plan_st(c, b, R);
+    if (b.L.nz > 1 || c->opts.tile_rows > 0 || c->ty_override > 0 || L.ty < 32) return L;
+    const int ty = spmv_wave_rows(R.j1 - L.jstart, R.k1 - R.k0);
+    // one reduction partial per CTA must fit the block's scratch (fewer CTAs: always true)
+    return plan_stencil(R, ty, 0);
+}
 // pointwise kernels: the 2D tiling of one plane, planes on grid.z
 Launch plan_pw(tea_ctx *c, const BlockCtx &b, const Region &R) {
     Launch L = plan(c, R);
@@ -460,7 +468,7 @@ double sbytes(const BlockCtx &b, int streams) {
 void body_cg(tea_ctx *c, int par, bool last_sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
-        Launch L = plan_st(c, b, R);
+        Launch L = plan_spmv(c, b, R);
         K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[F_R0], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
@@ -617,7 +625,7 @@ void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
     const int zs = zs_field(c, s);
     for (auto &b : c->blocks) {
         Region R = b.owned();
-        Launch L = plan_st(c, b, R);
+        Launch L = plan_spmv(c, b, R);
         K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[zs], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
@@ -642,7 +650,7 @@ void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
 void body_bj(tea_ctx *c, int par, bool sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
-        Launch L = plan_st(c, b, R);
+        Launch L = plan_spmv(c, b, R);
         K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[F_Z0], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);

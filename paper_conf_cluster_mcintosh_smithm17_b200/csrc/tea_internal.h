@@ -89,6 +89,7 @@ Launch plan_stencil(const Region &R, int ty_req, int ncta_target);
 // 3D stencil geometry: CTA = 4 warps on 4 consecutive rows of one 64-column strip,
 // marching tz planes (grid = strips x rows/4 x planes/tz).
 Launch plan_stencil3(const Region &R, int nz, int tz_req);
+int spmv_wave_rows(int width, int height);  // wave-fitted SpMV tile height (large blocks)
 int max_ctas3(int width, int height, int nz);
 Launch plan_pointwise(const Region &R, int ty_req, int ncta_target);
 int max_ctas(int width, int height);

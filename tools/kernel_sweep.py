@@ -40,7 +40,7 @@ def main():
         kt = t.kernel_times()
         t.close()
         row = {}
-        for k, (ms, n) in kt.items():
+        for k, (ms, n, *_) in kt.items():
             if n == 0:
                 continue
             us = 1e3 * ms / n
