@@ -286,7 +286,7 @@ def run_gpu(args):
     cells = args.n * args.n * max(args.nz, 1)
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
                 tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode,
-                persist=args.persist)
+                persist=args.persist, overlap=args.overlap)
     stream = t.stream
 
     def solve():
@@ -430,6 +430,10 @@ def main():
     ap.add_argument("--persist", type=int, default=0,
                     help="whole solve in one cooperative launch: 1 on, 0 (auto) or -1 off "
                          "(tea_opts.persist)")
+    ap.add_argument("--overlap", type=int, default=0,
+                    help="halo exchange of the fused passes overlapped with the interior on "
+                         "a second stream: 1 on, -1 off, 0 auto = on across processes "
+                         "(tea_opts.overlap)")
     ap.add_argument("--tb-steps", type=int, default=0,
                     help="Chebyshev steps per fused HBM pass (0 auto=4, 1 = per-step kernels)")
     ap.add_argument("--loop-mode", type=int, default=0,

@@ -31,7 +31,7 @@
 extern "C" {
 #endif
 
-#define TEA_ABI_VERSION 2
+#define TEA_ABI_VERSION 3
 
 typedef enum {
     TEA_OK = 0,
@@ -102,8 +102,9 @@ typedef struct {
     int profile;            /* 1: eager launches timed per kernel (tea_kernel_times)[0]*/
     int tile_rows;          /* rows per CTA tile of the stencil kernels, 0 = auto [0]  */
     int tb_steps;           /* Chebyshev steps fused per HBM pass (on-chip matrix
-                               powers, single block only): 0 = auto, 1 = one kernel
-                               per step, 2..5 = at most that many            [0 = 4] */
+                               powers): 0 = auto (5 for 2D blocks >= 4e5 cells with
+                               one block or d >= s + 1, else 1), 1 = one kernel per
+                               step, 2..5 = at most that many                [0]   */
     int tb_rows;            /* output rows per CTA tile of the fused passes, 0 = auto */
     int persist;            /* whole solve in ONE cooperative launch (grid-wide barriers
                                between the phases; single 2D block, CG / CPPCG, one
@@ -111,6 +112,16 @@ typedef struct {
                                on for CG blocks <= TEA_PERSIST_AUTO_CG cells and
                                CPPCG blocks <= TEA_PERSIST_AUTO_CPPCG cells, where it
                                measured faster              [0] */
+    int overlap;            /* with neighbour blocks and the fused passes (d >= s + 1):
+                               the residual's halo exchange runs on a second stream while
+                               the first pass computes the block interior that needs no
+                               halo cell; the frame follows the exchange (SURVEY §8(e)
+                               "Overlap"). 1 = on, -1 = off, 0 = auto:
+                               on when the halo crosses processes (nranks > 1; with all
+                               blocks in one process the copies are on-device and the
+                               split only adds launches: measured 383 vs 341 ms per
+                               4096^2 timestep in 2 x 4). Never while profiling. Results
+                               are bitwise identical either way.                [0] */
 } tea_opts;
 #define TEA_PERSIST_AUTO_CG (1024.0 * 1024.0)
 #define TEA_PERSIST_AUTO_CPPCG (512.0 * 512.0)

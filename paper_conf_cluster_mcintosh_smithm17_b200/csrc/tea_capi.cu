@@ -127,6 +127,9 @@ struct tea_ctx {
     std::vector<BlockCtx> blocks;
     cudaStream_t user_stream = nullptr, stream = nullptr;
     cudaEvent_t ev_in = nullptr, ev_t0 = nullptr, ev_t1 = nullptr;
+    // halo/compute overlap (tea_opts.overlap): exchange stream and its fork/join events
+    cudaStream_t xstream = nullptr;
+    cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
     Scalars *hS = nullptr;  // pinned host mirror (head only)
     ncclComm_t comm = nullptr;
     std::string err;
@@ -275,8 +278,11 @@ void reduce(tea_ctx *c, int first, int n) {
 }
 
 // ------------------------------------------------------------------ halo exchange
-void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field) {
-    // fids: field ids (same for every block), 1 or 2 entries
+void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field,
+              cudaStream_t xs = nullptr) {
+    // fids: field ids (same for every block), 1 or 2 entries; xs: the stream to run on
+    // (default: the compute stream)
+    const cudaStream_t st = xs ? xs : c->stream;
     const int nb = (int)c->blocks.size();
     if (c->px * c->py == 1) return;
     const int nf = (int)fids_per_block_field.size();
@@ -286,7 +292,7 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
         const double *F[4];
         for (int i = 0; i < nf; ++i) F[i] = b.f[fids_per_block_field[i]];
         K(c, TEA_K_PACK, 0.0, [&] {
-            launch_pack(F, nf, b.L.pitch, x.d_send, x.nsend, b.sendbuf, c->stream);
+            launch_pack(F, nf, b.L.pitch, x.d_send, x.nsend, b.sendbuf, st);
         });
     }
     // transport
@@ -314,12 +320,12 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
                     fail(TEA_ERR_STATE, "halo size mismatch %zu vs %zu", x.slen[d], y.rlen[od]);
                 CK(cudaMemcpyAsync(nbk.recvbuf + y.roff[od], b.sendbuf + x.soff[d],
                                    x.slen[d] * sizeof(double), cudaMemcpyDeviceToDevice,
-                                   c->stream));
+                                   st));
             } else {
                 NK(ncclSend(b.sendbuf + x.soff[d], x.slen[d], ncclDouble, nrank, c->comm,
-                            c->stream));
+                            st));
                 NK(ncclRecv(b.recvbuf + x.roff[d], x.rlen[d], ncclDouble, nrank, c->comm,
-                            c->stream));
+                            st));
             }
         }
     }
@@ -330,7 +336,7 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
         double *F[4];
         for (int i = 0; i < nf; ++i) F[i] = b.f[fids_per_block_field[i]];
         K(c, TEA_K_UNPACK, 0.0, [&] {
-            launch_unpack(F, nf, b.L.pitch, x.d_recv, x.nrecv, b.recvbuf, c->stream);
+            launch_unpack(F, nf, b.L.pitch, x.d_recv, x.nrecv, b.recvbuf, st);
         });
     }
     (void)nb;
@@ -561,7 +567,23 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
     const auto passes = tb_passes(s, tb_steps(c));
     const int pairA[2] = {F_Z0, F_Z2}, pairB[2] = {F_Z1, F_Z3};
     const bool blocks = !single_block(c);
-    if (blocks) exchange(c, X_RD, {rin});  // depth d >= s + 1, with corners
+    // Overlap: the depth-d exchange of r runs on the exchange stream while
+    // the first pass computes, on the compute stream, every output cell whose inputs
+    // (M rows / columns around it) are owned cells; the frame of the extended region
+    // follows the exchange. The first pass must not be the last (its dot products are one
+    // grid reduction); profiling keeps every launch on the compute stream.
+    const bool want = c->opts.overlap > 0 || (c->opts.overlap == 0 && c->nranks > 1);
+    const bool ovl = blocks && c->xstream && want && !c->profiling && passes.size() > 1;
+    if (blocks) {
+        if (ovl) {
+            CK(cudaEventRecord(c->ev_fork, c->stream));
+            CK(cudaStreamWaitEvent(c->xstream, c->ev_fork, 0));
+            exchange(c, X_RD, {rin}, c->xstream);  // depth d >= s + 1, with corners
+            CK(cudaEventRecord(c->ev_join, c->xstream));
+        } else {
+            exchange(c, X_RD, {rin});
+        }
+    }
     int step0 = 1, after = s;
     const int r = fused ? rout : rin;
     for (size_t p = 0; p < passes.size(); ++p) {
@@ -570,8 +592,42 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
         const bool first = p == 0, last = p + 1 == passes.size();
         const bool fu = fused && first;
         const int o = p % 2, in = (p + 1) % 2;
-        for (auto &b : c->blocks) {
+        // the regions this pass is launched on, per block: the whole (extended) region, or
+        // for the overlapped first pass the halo-free interior now and the frame after the
+        // exchange has landed
+        std::vector<std::vector<Region>> regs(c->blocks.size());
+        std::vector<std::vector<Region>> frame(c->blocks.size());
+        for (size_t i = 0; i < c->blocks.size(); ++i) {
+            const BlockCtx &b = c->blocks[i];
             const Region R = blocks ? b.ext(1 + after) : b.owned();
+            if (!(ovl && first)) {
+                regs[i].push_back(R);
+                continue;
+            }
+            const Region O = b.owned();
+            Region I{b.nbr[0] >= 0 ? O.j0 + M : R.j0, b.nbr[1] >= 0 ? O.j1 - M : R.j1,
+                     b.nbr[2] >= 0 ? O.k0 + M : R.k0, b.nbr[3] >= 0 ? O.k1 - M : R.k1};
+            if (I.j0 >= I.j1 || I.k0 >= I.k1) {
+                frame[i].push_back(R);  // block too small for an interior: all after
+                continue;
+            }
+            regs[i].push_back(I);
+            auto add = [&](Region q) {
+                if (q.j0 < q.j1 && q.k0 < q.k1) frame[i].push_back(q);
+            };
+            add(Region{R.j0, R.j1, R.k0, I.k0});  // bottom band (full width)
+            add(Region{R.j0, R.j1, I.k1, R.k1});  // top band
+            add(Region{R.j0, I.j0, I.k0, I.k1});  // west strip
+            add(Region{I.j1, R.j1, I.k0, I.k1});  // east strip
+        }
+        for (int phase = 0; phase < 2; ++phase) {
+          if (phase == 1) {
+              if (!(ovl && first)) break;
+              CK(cudaStreamWaitEvent(c->stream, c->ev_join, 0));
+          }
+          for (size_t i = 0; i < c->blocks.size(); ++i)
+          for (const Region &R : (phase == 0 ? regs[i] : frame[i])) {
+            auto &b = c->blocks[i];
             const Region D = b.owned();
             const int jlim = b.L.pitch - b.L.X0;
             int ty = c->opts.tb_rows > 0 ? c->opts.tb_rows : 0;
@@ -591,6 +647,7 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
                                first ? nullptr : b.f[pairA[in]], b.f[pairA[o]], b.f[pairB[o]],
                                b.f[F_KX], b.f[F_KY], c->stream);
             });
+          }
         }
         step0 += M;
     }
@@ -1136,6 +1193,7 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
         }
         if (o.loop_mode < 0 || o.loop_mode > 2) fail(TEA_ERR_ARG, "bad loop_mode");
         if (o.persist < -1 || o.persist > 1) fail(TEA_ERR_ARG, "bad persist");
+        if (o.overlap < -1 || o.overlap > 1) fail(TEA_ERR_ARG, "bad overlap");
         // NCCL kernels inside a WHILE-conditional graph body are not a supported
         // capture target: multi-process runs use chunked graphs (same kernels).
         if (nranks > 1 && o.loop_mode == 0) o.loop_mode = 1;
@@ -1149,6 +1207,11 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
         CK(cudaEventCreateWithFlags(&c->ev_in, cudaEventDisableTiming));
         CK(cudaEventCreate(&c->ev_t0));
         CK(cudaEventCreate(&c->ev_t1));
+        if (px * py > 1) {
+            CK(cudaStreamCreateWithFlags(&c->xstream, cudaStreamNonBlocking));
+            CK(cudaEventCreateWithFlags(&c->ev_fork, cudaEventDisableTiming));
+            CK(cudaEventCreateWithFlags(&c->ev_join, cudaEventDisableTiming));
+        }
         CK(cudaMallocHost((void **)&c->hS, sizeof(Scalars)));
         std::memset(c->hS, 0, sizeof(Scalars));
         CK(cudaEventRecord(c->ev_in, c->user_stream));
@@ -1332,6 +1395,9 @@ tea_status tea_finalize(tea_ctx *ctx) {
     if (ctx->ev_in) cudaEventDestroy(ctx->ev_in);
     if (ctx->ev_t0) cudaEventDestroy(ctx->ev_t0);
     if (ctx->ev_t1) cudaEventDestroy(ctx->ev_t1);
+    if (ctx->ev_fork) cudaEventDestroy(ctx->ev_fork);
+    if (ctx->ev_join) cudaEventDestroy(ctx->ev_join);
+    if (ctx->xstream) cudaStreamDestroy(ctx->xstream);
     if (ctx->hS) cudaFreeHost(ctx->hS);
     if (ctx->comm) ncclCommDestroy(ctx->comm);
     if (ctx->stream) cudaStreamDestroy(ctx->stream);

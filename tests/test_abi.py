@@ -50,8 +50,15 @@ def test_sm100a_sass():
 
 
 def test_version(L):
+    import re
     assert "sm_100a" in tea.version()
-    assert L.tea_abi_version() == 2
+    hdr = open(os.path.join(ROOT, "include", "tea.h")).read()
+    v = int(re.search(r"#define TEA_ABI_VERSION (\d+)", hdr).group(1))
+    assert L.tea_abi_version() == v == tea.ABI_VERSION
+    # the binding's tea_opts mirrors the header's field list (same order)
+    body = hdr[hdr.index("typedef struct {", hdr.index("Solver options")):hdr.index("} tea_opts;")]
+    fields = re.findall(r"^\s+(?:int|double)\s+(\w+);", body, re.M)
+    assert fields == [f for f, _ in tea.Opts._fields_]
 
 
 @pytest.mark.parametrize("nx,ny,px,py", [(4096, 4096, 2, 4), (1000, 777, 3, 2), (17, 5, 4, 1),

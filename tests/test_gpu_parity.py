@@ -532,6 +532,37 @@ def test_fused_passes_blocks_fixed_iterations(tea, ora):
     assert field_err(u_g, u_o, "random") <= 1e-12
 
 
+@pytest.mark.parametrize("nx,ny,px,py,d,s,tb", [(240, 200, 2, 2, 11, 10, 5),
+                                                (201, 143, 3, 2, 12, 10, 4),
+                                                (150, 90, 1, 3, 6, 5, 3),
+                                                (36, 24, 3, 2, 11, 10, 5)])
+@pytest.mark.parametrize("loop_mode", [0, 1, 2])
+def test_overlap_bitwise(tea, nx, ny, px, py, d, s, tb, loop_mode):
+    """Halo/compute overlap (tea_opts.overlap): the first fused pass split
+    into the halo-free interior (concurrent with the exchange on the second stream) and the
+    frame after it gives bitwise the same fields and scalars as the unsplit pass, down to
+    the smallest legal blocks (12 x 12 at d = 11: a 2 x 2 interior)."""
+    deck = deck_of("random", nx, ny, seed=nx * ny, dt=0.04)
+    kw = dict(method=1, eps=0.0, max_iters=30 + 6, inner_steps=s, tb_steps=tb,
+              loop_mode=loop_mode, dist=dict(px=px, py=py, halo_depth=d, nranks=1))
+    u_a, st_a = gpu_run(tea, deck, overlap=1, **kw)
+    u_b, st_b = gpu_run(tea, deck, overlap=-1, **kw)
+    assert st_a[0]["iterations"] == st_b[0]["iterations"] == 36
+    assert np.array_equal(u_a, u_b)
+    assert st_a[0]["rnorm"] == st_b[0]["rnorm"]
+
+
+def test_overlap_converged_against_oracle(tea, ora):
+    deck = deck_of("pipe", 256, 192)
+    kw = dict(method=1, eps=1e-13, max_iters=20000, inner_steps=10)
+    u_o, st_o, _ = ora.run(deck, steps=2, **kw)
+    u_g, st_g = gpu_run(tea, deck, steps=2, dist=dict(px=2, py=2, halo_depth=11, nranks=1),
+                        tb_steps=5, overlap=1, **kw)
+    for a, b in zip(st_g, st_o):
+        assert a["ret"] == 0 and abs(a["iterations"] - b["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+
+
 # ---------------------------------------------------------------- persistent solver
 # tea_opts.persist = 1: the whole solve in ONE cooperative launch (k_persist, grid-wide
 # barriers between the phases; DESIGN.md §4.12). Same device bodies as the graph path.

@@ -20,9 +20,15 @@ def main():
         # persistent solver (one cooperative launch; needs the device-loop mode)
         (inputs.crooked_pipe(96, 70), None, dict(persist=1, loop_mode=0)),
         (inputs.random_fields(300, 41, 5), None, dict(persist=1, loop_mode=0, tile_rows=1)),
+        # fused passes across blocks with the halo exchange overlapped (second stream)
+        (inputs.random_fields(90, 60, 4), dict(px=2, py=2, halo_depth=11, nranks=1),
+         dict(tb_steps=5, overlap=1, _s=10, _methods=(1,))),
     ]
     for deck, dist, kw in cases:
-        for method in (0, 1, 2, 3, 4, 5):
+        kw = dict(kw)
+        s = kw.pop("_s", 4)
+        methods = kw.pop("_methods", (0, 1, 2, 3, 4, 5))
+        for method in methods:
             if getattr(deck, "nz", 1) > 1 and method == 2:
                 continue
             if kw.get("persist") and method > 1:
@@ -30,7 +36,7 @@ def main():
             kw = dict(dict(loop_mode=2, check_interval=4), **kw)
             t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist,
                         presteps=10, **kw)
-            r = t.solve(method, 1e-10, 60, 4, raise_on_error=False)
+            r = t.solve(method, 1e-10, 60, s, raise_on_error=False)
             t.fetch()
             t.close()
             print(deck.name, dist, kw, method, r.status, r.stats["iterations"], flush=True)
