@@ -256,7 +256,11 @@ Launch plan_spmv(tea_ctx *c, const BlockCtx &b, const Region &R) {
 }
 // pointwise kernels: the 2D tiling of one plane, planes on grid.z
 Launch plan_pw(tea_ctx *c, const BlockCtx &b, const Region &R) {
-    Launch L = plan(c, R);
+    // 3D: the planes already multiply the CTA count, so the small-block rule of
+    // plan_stencil (shorter tiles until >= 2 tiles per SM, a 2D latency fix) must not
+    // apply: it cut 256^3 tiles to one row (CG 67 -> 85 ms per timestep). 8-row tiles.
+    const int tr = c->opts.tile_rows > 0 ? c->opts.tile_rows : c->ty_override;
+    Launch L = b.L.nz > 1 ? plan_stencil(R, tr > 0 ? tr : 8, 1184) : plan(c, R);
     L.grid.z = b.L.nz;
     return L;
 }
