@@ -143,7 +143,8 @@ def run_reference(args):
     oracle.build()
     deck = make_deck(args)
     method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
-              "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY}[args.method]
+              "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY,
+              "cppcg1": oracle.CPPCG1}[args.method]
     sample_iters = args.ref_iters
     orun = oracle.run3 if args.nz > 1 else oracle.run
     for _ in range(args.warmup):  # untimed warm-up (page-in, caches)
@@ -176,7 +177,8 @@ def run_reference(args):
 
 
 METHOD_NAME = {"cppcg": "CPPCG", "cg": "CG", "bjcg": "block-Jacobi PCG",
-               "cg1": "single-reduction CG", "jacobi": "Jacobi", "cheby": "Chebyshev"}
+               "cg1": "single-reduction CG", "jacobi": "Jacobi", "cheby": "Chebyshev",
+               "cppcg1": "single-reduction CPPCG"}
 
 
 def make_deck(args):
@@ -213,7 +215,8 @@ def cpu_baseline(args, deck):
     import oracle
     oracle.build()
     method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
-              "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY}[args.method]
+              "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY,
+              "cppcg1": oracle.CPPCG1}[args.method]
     t0 = time.perf_counter()
     orun = oracle.run3 if args.nz > 1 else oracle.run
     _, st, _ = orun(deck, steps=1, method=method, eps=args.eps, max_iters=args.ref_iters,
@@ -282,7 +285,8 @@ def run_gpu(args):
         dist_kw = dict(rank=0, nranks=1, px=bpx, py=bpy, halo_depth=args.halo_depth)
     deck = make_deck(args)
     method = {"cppcg": tea.CPPCG, "cg": tea.CG, "bjcg": tea.BJCG,
-              "cg1": tea.CG1, "jacobi": tea.JACOBI, "cheby": tea.CHEBY}[args.method]
+              "cg1": tea.CG1, "jacobi": tea.JACOBI, "cheby": tea.CHEBY,
+              "cppcg1": tea.CPPCG1}[args.method]
     cells = args.n * args.n * max(args.nz, 1)
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
                 tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode,
@@ -317,6 +321,12 @@ def run_gpu(args):
         model_bytes = sum(5 * 8 * cells + s["presteps"] * cg_iter_bytes(cells) +
                           outer_bytes(cells, args.inner) - 10 * 8 * cells +  # restart chain
                           s["outer"] * outer_bytes(cells, args.inner) for s in stats)
+    elif method == tea.CPPCG1:
+        # per outer: update 10 + q = A z 4 + the chain priced at one kernel per step
+        chain_st = 4 if args.inner == 1 else 4 + 5 + 6 * (args.inner - 2)
+        model_bytes = sum(5 * 8 * cells + s["presteps"] * cg_iter_bytes(cells) +
+                          (chain_st + 4) * 8 * cells + s["outer"] * (10 + 4 + chain_st) * 8 * cells
+                          for s in stats)
     elif method in (tea.JACOBI, tea.CHEBY):
         per = 5 if method == tea.JACOBI else 6
         model_bytes = len(stats) * 5 * 8 * cells + iters * per * 8 * cells
@@ -414,7 +424,8 @@ def main():
     ap.add_argument("--n", type=int, default=4096)
     ap.add_argument("--nz", type=int, default=0,
                     help="> 1: the 3D 7-point problem on n x n x nz (SURVEY NEXT-4)")
-    ap.add_argument("--method", default="cppcg", choices=["cppcg", "cg", "bjcg", "cg1", "jacobi", "cheby"])
+    ap.add_argument("--method", default="cppcg", choices=["cppcg", "cg", "bjcg", "cg1", "jacobi", "cheby",
+                                                   "cppcg1"])
     ap.add_argument("--inner", type=int, default=10)
     ap.add_argument("--eps", type=float, default=1e-12)
     ap.add_argument("--max-iters", type=int, default=0,
@@ -444,7 +455,7 @@ def main():
     if args.warmup < 3:
         ap.error("--warmup must be >= 3")
     if args.halo_depth == 0:
-        args.halo_depth = args.inner + 1 if args.method == "cppcg" else 1
+        args.halo_depth = args.inner + 1 if args.method in ("cppcg", "cppcg1") else 1
     if args.max_iters == 0:
         args.max_iters = 2000 if args.method in ("jacobi", "cheby") else 100000
     if args.impl == "reference":

@@ -51,6 +51,13 @@ typedef enum {
  * reduction per iteration, s = A p carried by recurrence -- the restructuring the
  * paper names as future work. Same iterates as CG in
  * exact arithmetic; one fused kernel per iteration on a single block.             */
+/* TEA_CPPCG1: single-reduction CPPCG: the same presteps, eigen-estimate and Chebyshev
+ * preconditioner B(A) as TEA_CPPCG, with the outer PCG in Chronopoulos & Gear's form:
+ * q = A z and s = A p carried by recurrence, so r.z, z.q and r.r form ONE global
+ * reduction per outer iteration instead of two (P:L817-821 applied to CPPCG; SURVEY
+ * NEXT-2). Same iterates as CPPCG in exact arithmetic; one more matvec per outer
+ * iteration (q = A z) and a separate pointwise update, so on one GPU it moves more bytes
+ * than TEA_CPPCG -- its point is the halved allreduce count across ranks.            */
 /* TEA_JACOBI / TEA_CHEBY: the stand-alone solvers TeaLeaf ships beside CG
  * (SURVEY NEXT-4): point Jacobi u += D^{-1} (u^n - A u), and the Chebyshev
  * iteration (Saad Alg. 12.1) on the interval estimated from `presteps` CG iterations
@@ -58,7 +65,8 @@ typedef enum {
  * the iterate before the last update (reading R19). Chebyshev "cannot cope with some
  * condition numbers": max_iters bounds it.                          */
 typedef enum {
-    TEA_CG = 0, TEA_CPPCG = 1, TEA_BJCG = 2, TEA_CG1 = 3, TEA_JACOBI = 4, TEA_CHEBY = 5
+    TEA_CG = 0, TEA_CPPCG = 1, TEA_BJCG = 2, TEA_CG1 = 3, TEA_JACOBI = 4, TEA_CHEBY = 5,
+    TEA_CPPCG1 = 6
 } tea_method;
 
 typedef struct tea_ctx tea_ctx; /* opaque, library-owned */

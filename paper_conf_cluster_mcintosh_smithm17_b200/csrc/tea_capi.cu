@@ -499,7 +499,8 @@ void body_cg(tea_ctx *c, int par, bool last_sets_cond) {
 // Chebyshev chain z = B(A) r, one kernel per step (blocks with neighbours; or
 // tb_steps == 1). fused: the first step also does r_out = r_in - alpha w (single
 // block only). Returns the field holding z_s.
-int cheb_chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond) {
+int cheb_chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond,
+               bool reduce_dots = true) {
     auto ops = cheb_schedule(s, c->d);
     int r = fused ? rout : rin;
     int step = 0;
@@ -530,7 +531,7 @@ int cheb_chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, b
                                 b.f[zbuf(step)], b.f[F_KX], b.f[F_KY], c->stream);
                 });
             }
-            if (last) reduce(c, 1, 2);
+            if (last && reduce_dots) reduce(c, 1, 2);
         }
     }
     return zbuf(s);
@@ -567,7 +568,7 @@ bool is3d(const tea_ctx *c) { return c->blocks[0].L.nz > 1; }
 // 1 + (steps after it), so the last pass leaves z_s valid on the 1-cell ring the next
 // SpMV reads; no z exchange. (One block: every extension is empty.)
 int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout,
-                  bool sets_cond) {
+                  bool sets_cond, bool reduce_dots = true) {
     const auto passes = tb_passes(s, tb_steps(c));
     const int pairA[2] = {F_Z0, F_Z2}, pairB[2] = {F_Z1, F_Z3};
     const bool blocks = !single_block(c);
@@ -655,7 +656,7 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
         }
         step0 += M;
     }
-    reduce(c, 1, 2);
+    if (reduce_dots) reduce(c, 1, 2);
     return pairB[(passes.size() - 1) % 2];
 }
 
@@ -667,9 +668,13 @@ bool use_tb(tea_ctx *c, int s) {
     return single_block(c) || c->d >= s + 1;
 }
 
-int chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond) {
-    if (use_tb(c, s)) return cheb_chain_tb(c, s, restart, fused, rin, rout, sets_cond);
-    return cheb_chain(c, s, restart, fused, rin, rout, sets_cond);
+// reduce_dots = false: the caller folds the chain's [r.z, r.r] into its own single
+// reduction (single-reduction CPPCG)
+int chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool sets_cond,
+          bool reduce_dots = true) {
+    if (use_tb(c, s))
+        return cheb_chain_tb(c, s, restart, fused, rin, rout, sets_cond, reduce_dots);
+    return cheb_chain(c, s, restart, fused, rin, rout, sets_cond, reduce_dots);
 }
 
 // field holding z_s after a chain (same for every chain of a context and s)
@@ -759,6 +764,33 @@ void body_cg1(tea_ctx *c, int par, bool sets_cond) {
         K(c, TEA_K_CG1W, sbytes(b, 4), [&] {
             launch_cg1_w(kargs(c, b, sets_cond), L, R, b.f[F_R0], b.f[F_Z0], b.f[F_KX],
                          b.f[F_KY], c->stream);
+        });
+    }
+    reduce(c, 0, 3);
+}
+
+// Single-reduction CPPCG outer iteration (Chronopoulos-Gear PCG with M^-1 = B(A); oracle
+// ORA_CPPCG1): pointwise update (alpha, beta from the last reduction; p = z + b p,
+// s = q + b s, u += a p, r -= a s) -> Chebyshev chain z = B(A) r with r.z, r.r (no
+// reduction of its own) -> q = A z with z.q -> ONE reduction of [z.q, r.z, r.r].
+// Fields: z in zs_field, q in W, s in R1, p in P0 (no ping-pong: the update is pointwise).
+void body_pcg1(tea_ctx *c, int s, int /*par*/, bool sets_cond) {
+    const int zs = zs_field(c, s);
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan_pw(c, b, R);
+        K(c, TEA_K_UPDATE, sbytes(b, 10), [&] {
+            launch_cg1_update(kargs(c, b), L, R, b.f[F_W], b.f[F_R1], b.f[F_P0], b.f[F_U],
+                              b.f[F_R0], c->stream, b.f[zs]);
+        });
+    }
+    chain(c, s, false, false, F_R0, F_R0, false, false);
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan_st(c, b, R);
+        K(c, TEA_K_CG1W, sbytes(b, 4), [&] {
+            launch_cg1_w(kargs(c, b, sets_cond), L, R, b.f[zs], b.f[F_W], b.f[F_KX], b.f[F_KY],
+                         c->stream, true);
         });
     }
     reduce(c, 0, 3);
@@ -933,13 +965,14 @@ void solve_persist(tea_ctx *c, int s, bool two_phase) {
 tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, int s,
                       tea_stats *st) {
     if (c->failed) fail(TEA_ERR_STATE, "context already failed: %s", c->err.c_str());
-    if (method < TEA_CG || method > TEA_CHEBY) fail(TEA_ERR_ARG, "bad method %d", (int)method);
+    if (method < TEA_CG || method > TEA_CPPCG1) fail(TEA_ERR_ARG, "bad method %d", (int)method);
     if (method == TEA_BJCG && is3d(c)) fail(TEA_ERR_ARG, "block Jacobi is 2D only");
     if (max_iters < 0) fail(TEA_ERR_ARG, "max_iters < 0");
-    if (method == TEA_CPPCG && (s < 1 || s > kMaxS))
+    const bool pcg = method == TEA_CPPCG || method == TEA_CPPCG1;
+    if (pcg && (s < 1 || s > kMaxS))
         fail(TEA_ERR_ARG, "inner_steps must be in [1,%d]", kMaxS);
     const int pre = c->opts.presteps;
-    if ((method == TEA_CPPCG || method == TEA_CHEBY) && (pre < 1 || pre > kMaxPre))
+    if ((pcg || method == TEA_CHEBY) && (pre < 1 || pre > kMaxPre))
         fail(TEA_ERR_ARG, "presteps must be in [1,%d]", kMaxPre);
     c->profiling = c->opts.profile != 0;
 
@@ -947,7 +980,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
     CK(cudaStreamWaitEvent(c->stream, c->ev_in, 0));
     CK(cudaEventRecord(c->ev_t0, c->stream));
 
-    const bool two_phase = method == TEA_CPPCG || method == TEA_CHEBY;
+    const bool two_phase = pcg || method == TEA_CHEBY;
     const int lim1 = two_phase ? std::min(pre, max_iters) : max_iters;
     for (auto &b : c->blocks)
         K(c, TEA_K_SCALAR, 0.0, [&] {
@@ -1040,11 +1073,30 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         // the fused passes read the coefficients from constant memory (every block's copy
         // is identical: they derive from globally reduced scalars)
         if (use_tb(c, s)) CK(tb_coef_upload(c->coef_slot, c->blocks[0].S, c->stream));
-        chain(c, s, true, false, F_R0, F_R0, false);
+        if (method == TEA_CPPCG1) {
+            // z = B(A) r, q = A z, [z.q, r.z, r.r] in one reduction; p = s = 0 (b_0 = 0)
+            chain(c, s, true, false, F_R0, F_R0, false, false);
+            const int zs = zs_field(c, s);
+            for (auto &b : c->blocks) {
+                Region R = b.owned();
+                Launch L = plan_st(c, b, R);
+                K(c, TEA_K_CG1W, sbytes(b, 4), [&] {
+                    launch_cg1_w(kargs(c, b), L, R, b.f[zs], b.f[F_W], b.f[F_KX], b.f[F_KY],
+                                 c->stream, true);
+                });
+            }
+            reduce(c, 0, 3);
+        } else {
+            chain(c, s, true, false, F_R0, F_R0, false);
+        }
         read_state(c);
         if (!c->hS->done) {
-            long long key = 2 + 16LL * s;
-            run_loop(c, key, max_iters, [&](int par, bool sc) { body_pcg(c, s, par, sc); });
+            if (method == TEA_CPPCG1)
+                run_loop(c, 7 + 16LL * s, max_iters,
+                         [&](int par, bool sc) { body_pcg1(c, s, par, sc); });
+            else
+                run_loop(c, 2 + 16LL * s, max_iters,
+                         [&](int par, bool sc) { body_pcg(c, s, par, sc); });
         }
         ds = c->hS->status;
     }
@@ -1062,8 +1114,9 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         st->iterations = h.it;
         st->presteps = phase2 ? h.presteps : 0;
         st->outer = phase2 ? h.outer : 0;
-        st->inner_matvecs = phase2 && method == TEA_CPPCG ? s * (h.outer + 1) : 0;
-        st->matvecs = 1 + h.it + st->inner_matvecs + (method == TEA_CG1 ? 1 : 0);
+        st->inner_matvecs = phase2 && pcg ? s * (h.outer + 1) : 0;
+        st->matvecs = 1 + h.it + st->inner_matvecs + (method == TEA_CG1 ? 1 : 0) +
+                      (phase2 && method == TEA_CPPCG1 ? 1 : 0);
         st->status = rs;
         st->r0 = h.r0;
         st->rnorm = std::sqrt(h.red_rr);

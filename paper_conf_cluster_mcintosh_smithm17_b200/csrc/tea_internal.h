@@ -151,10 +151,13 @@ void launch_cg1(const KArgs &a, const Launch &L, const Region &R, const double *
                 const double *win, const double *sin, double *rout, double *wout, double *sout,
                 double *p, double *u, const double *kx, const double *ky, cudaStream_t st);
 // Multi-block: pointwise update (s, p, u, r) then w = A r with the dots.
+// z == nullptr: CG1 (p = r + b p, counts the iteration); else CPPCG1 (p = z + b p)
 void launch_cg1_update(const KArgs &a, const Launch &L, const Region &R, const double *w,
-                       double *s, double *p, double *u, double *r, cudaStream_t st);
+                       double *s, double *p, double *u, double *r, cudaStream_t st,
+                       const double *z = nullptr);
+// pw_only: w = A r and red_pw = r.w only (CPPCG1's q = A z, del = z.q)
 void launch_cg1_w(const KArgs &a, const Launch &L, const Region &R, const double *r, double *w,
-                  const double *kx, const double *ky, cudaStream_t st);
+                  const double *kx, const double *ky, cudaStream_t st, bool pw_only = false);
 
 // Temporally blocked Chebyshev passes (tea_cheb_tb.cu).
 constexpr int kTbMaxSteps = 5;

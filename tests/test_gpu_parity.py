@@ -385,7 +385,55 @@ def test_cg1_multiblock(tea, ora, px, py):
     assert rel_err(u_g, u_o) <= 1e-10
 
 
-@pytest.mark.parametrize("method", [2, 3])
+# ---------------------------------------------------------------- single-reduction CPPCG
+@pytest.mark.parametrize("kind,nx,ny,s,tb", [("pipe", 128, 128, 10, 0), ("pipe", 256, 200, 10, 5),
+                                             ("pipe", 256, 200, 10, 1), ("random", 300, 203, 4, 0),
+                                             ("random", 97, 61, 3, 0), ("random", 1000, 777, 10, 0)])
+def test_cppcg1_converged(tea, ora, kind, nx, ny, s, tb):
+    """Single-reduction CPPCG (TEA_CPPCG1): converged solve against the oracle (+-2 outer
+    iterations, 1e-10), with the fused passes (tb 5, and auto at 1000 x 777) and with one
+    kernel per step (tb 1)."""
+    deck = deck_of(kind, nx, ny, seed=6)
+    kw = dict(method=6, eps=1e-13, max_iters=20000, inner_steps=s)
+    u_o, st_o, s_o = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, tb_steps=tb, **kw)
+    assert s_o[0] == 0 and st_g[0]["ret"] == 0
+    assert st_g[0]["presteps"] == st_o[0]["presteps"]
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert st_g[0]["matvecs"] == 1 + st_g[0]["iterations"] + s * (st_g[0]["outer"] + 1) + 1
+    assert field_err(u_g, u_o, kind) <= 1e-10
+    # same solution as CPPCG on the GPU, one reduction per outer iteration instead of two
+    u_c, st_c = gpu_run(tea, deck, tb_steps=tb, **dict(kw, method=1))
+    assert abs(st_c[0]["outer"] - st_g[0]["outer"]) <= 2
+    assert rel_err(u_g, u_c) <= 1e-10
+
+
+@pytest.mark.parametrize("k", [1, 2, 7])
+@pytest.mark.parametrize("tb", [1, 5])
+def test_cppcg1_fixed_iterations(tea, ora, k, tb):
+    deck = deck_of("random", 300, 203, seed=8, dt=0.04)
+    kw = dict(method=6, eps=0.0, max_iters=30 + k, inner_steps=10)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, tb_steps=tb, **kw)
+    assert st_g[0]["iterations"] == 30 + k and st_g[0]["outer"] == k
+    assert field_err(u_g, u_o, "random") <= 1e-12
+    assert st_g[0]["rnorm"] == pytest.approx(st_o[0]["rnorm"], rel=1e-9)
+
+
+@pytest.mark.parametrize("px,py,d,tb", [(2, 1, 11, 5), (2, 2, 11, 5), (1, 3, 2, 0), (4, 2, 4, 0)])
+@pytest.mark.parametrize("loop_mode", [0, 2])
+def test_cppcg1_multiblock(tea, ora, px, py, d, tb, loop_mode):
+    deck = deck_of("pipe", 200, 170)
+    kw = dict(method=6, eps=1e-13, max_iters=20000, inner_steps=10)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, dist=dict(px=px, py=py, halo_depth=d, nranks=1), tb_steps=tb,
+                        loop_mode=loop_mode, **kw)
+    assert st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+
+
+@pytest.mark.parametrize("method", [2, 3, 6])
 @pytest.mark.parametrize("loop_mode", [1, 2])
 def test_new_methods_loop_modes_identical(tea, method, loop_mode):
     deck = deck_of("pipe", 200, 136)
