@@ -22,16 +22,16 @@ def main():
         (inputs.random_fields(300, 41, 5), None, dict(persist=1, loop_mode=0, tile_rows=1)),
         # fused passes across blocks with the halo exchange overlapped (second stream)
         (inputs.random_fields(90, 60, 4), dict(px=2, py=2, halo_depth=11, nranks=1),
-         dict(tb_steps=5, overlap=1, _s=10, _methods=(1,))),
+         dict(tb_steps=5, overlap=1, _s=10, _methods=(1, 6))),
     ]
     for deck, dist, kw in cases:
         kw = dict(kw)
         s = kw.pop("_s", 4)
-        methods = kw.pop("_methods", (0, 1, 2, 3, 4, 5))
+        methods = kw.pop("_methods", (0, 1, 2, 3, 4, 5, 6))
         for method in methods:
             if getattr(deck, "nz", 1) > 1 and method == 2:
                 continue
-            if kw.get("persist") and method > 1:
+            if kw.get("persist") and method not in (0, 1):
                 continue
             kw = dict(dict(loop_mode=2, check_interval=4), **kw)
             t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist,
