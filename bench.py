@@ -204,7 +204,7 @@ def config(args):
             "mesh": [args.n, args.n] + ([args.nz] if args.nz > 1 else []),
             "method": args.method, "inner_steps": args.inner,
             "eps": args.eps, "max_iters": args.max_iters, "halo_depth": args.halo_depth,
-            "dt": 0.004,
+            "dt": 0.004, "kform": "stored Kx, Ky" if args.kform < 0 else "g = 1/rho on the fly",
             "l2": "inputs larger than L2 (>= 12 fp64 fields x 8 B x cells > 126 MB)"
             if args.n * args.n * max(args.nz, 1) >= 2 ** 21 else
             "working set fits in L2 (no flush)"}
@@ -290,7 +290,7 @@ def run_gpu(args):
     cells = args.n * args.n * max(args.nz, 1)
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
                 tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode,
-                persist=args.persist, overlap=args.overlap)
+                persist=args.persist, overlap=args.overlap, kform=args.kform)
     stream = t.stream
 
     def solve():
@@ -359,7 +359,7 @@ def run_gpu(args):
     # ---- roofline of the dominant kernel: profiled solve (events per launch)
     tp = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
                  profile=True, tile_rows=args.tile_rows, tb_steps=args.tb_steps,
-                 check_interval=2)
+                 check_interval=2, kform=args.kform)
     tp.set_u(u_np)
     pst = tp.solve(method, args.eps, args.max_iters, args.inner).stats
     kt = tp.kernel_times()
@@ -445,6 +445,9 @@ def main():
                     help="halo exchange of the fused passes overlapped with the interior on "
                          "a second stream: 1 on, -1 off, 0 auto = on across processes "
                          "(tea_opts.overlap)")
+    ap.add_argument("--kform", type=int, default=0,
+                    help="2D faces formed on the fly from g = 1/rho (1, auto 0) or read as stored "
+                         "Kx, Ky (-1) (tea_opts.kform)")
     ap.add_argument("--tb-steps", type=int, default=0,
                     help="Chebyshev steps per fused HBM pass (0 auto=4, 1 = per-step kernels)")
     ap.add_argument("--loop-mode", type=int, default=0,

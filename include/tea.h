@@ -31,7 +31,7 @@
 extern "C" {
 #endif
 
-#define TEA_ABI_VERSION 3
+#define TEA_ABI_VERSION 4
 
 typedef enum {
     TEA_OK = 0,
@@ -130,6 +130,14 @@ typedef struct {
                                split only adds launches: measured 383 vs 341 ms per
                                4096^2 timestep in 2 x 4). Never while profiling. Results
                                are bitwise identical either way.                [0] */
+    int kform;              /* face coefficients in the 2D SpMV and the fused Chebyshev
+                               passes: 1 = formed on the fly from ONE stream g = 1/rho
+                               (mean_mode 1: g = rho) as K = (r/2)(g_L + g_R) (reading
+                               R1 written out; one fp64 stream instead of the two
+                               stored Kx, Ky: 8 -> 7 and 7/6 -> 6/5 streams), -1 =
+                               stored Kx, Ky, 0 = auto (on). Every kernel's K is
+                               bitwise the same either way (the stored faces are
+                               computed by the same expression). [0] */
 } tea_opts;
 #define TEA_PERSIST_AUTO_CG (1024.0 * 1024.0)
 #define TEA_PERSIST_AUTO_CPPCG (512.0 * 512.0)

@@ -43,7 +43,7 @@ class Mesh(C.Structure):
                 ("zmin", C.c_double), ("zmax", C.c_double)]
 
 
-ABI_VERSION = 3  # include/tea.h TEA_ABI_VERSION (tea_opts layout)
+ABI_VERSION = 4  # include/tea.h TEA_ABI_VERSION (tea_opts layout)
 
 
 class Dist(C.Structure):
@@ -56,7 +56,7 @@ class Opts(C.Structure):
                 ("eig_margin_hi", C.c_double), ("mean_mode", C.c_int), ("loop_mode", C.c_int),
                 ("check_interval", C.c_int), ("profile", C.c_int), ("tile_rows", C.c_int),
                 ("tb_steps", C.c_int), ("tb_rows", C.c_int), ("persist", C.c_int),
-                ("overlap", C.c_int)]
+                ("overlap", C.c_int), ("kform", C.c_int)]
 
 
 class Stats(C.Structure):
@@ -181,7 +181,7 @@ class Tea:
                  presteps: int = 30, eig_margins=(0.95, 1.05), mean_mode: int = 0,
                  loop_mode: int = 0, check_interval: int = 0, profile: bool = False,
                  tile_rows: int = 0, tb_steps: int = 0, tb_rows: int = 0, persist: int = 0,
-                 overlap: int = 0, device=None, stream=None):
+                 overlap: int = 0, kform: int = 0, device=None, stream=None):
         import torch
         if not torch.cuda.is_available():
             raise RuntimeError("paper_conf_cluster_mcintosh_smithm17_b200 needs a CUDA device "
@@ -202,7 +202,7 @@ class Tea:
                               C.cast(self._nccl_id, C.c_void_p) if self._nccl_id else None)
         self.opts = Opts(presteps, eig_margins[0], eig_margins[1], mean_mode, loop_mode,
                          check_interval, 1 if profile else 0, tile_rows, tb_steps, tb_rows,
-                         persist, overlap)
+                         persist, overlap, kform)
         with torch.cuda.device(self.device):
             nbytes = workspace_bytes(mesh, self._dist)
             self.workspace = torch.empty(nbytes, dtype=torch.uint8, device=self.device)

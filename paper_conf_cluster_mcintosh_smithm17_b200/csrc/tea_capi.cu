@@ -196,6 +196,10 @@ KArgs kargs(tea_ctx *c, const BlockCtx &b, bool set_cond = false) {
     a.ps = b.L.ps;
     a.nz = b.L.nz;
     a.coef_slot = c->coef_slot;
+    // 2D blocks: faces formed on the fly from g (held in the otherwise unused Kz field)
+    a.g = (b.L.nz == 1 && c->opts.kform >= 0) ? b.f[F_KZ] : nullptr;
+    a.hrx = 0.5 * c->rx;
+    a.hry = 0.5 * c->ry;
     return a;
 }
 
@@ -474,12 +478,16 @@ double *field_base(const BlockCtx &b, int f) {
 double sbytes(const BlockCtx &b, int streams) {
     return 8.0 * streams * (double)b.L.bx * (double)b.L.by * (double)b.L.nz;
 }
+// face-coefficient streams of a 2D stencil launch: g alone (tea_opts.kform) or Kx + Ky
+int kstreams(const tea_ctx *c, const BlockCtx &b) {
+    return (b.L.nz == 1 && c->opts.kform >= 0) ? 1 : 2;
+}
 
 void body_cg(tea_ctx *c, int par, bool last_sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan_spmv(c, b, R);
-        K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
+        K(c, TEA_K_SPMV, sbytes(b, 6 + kstreams(c, b)), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[F_R0], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
         });
@@ -642,7 +650,7 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
             while (ty < R.k1 - R.k0 &&
                    2 * (size_t)tb_ctas(M, R.j1 - R.j0, R.k1 - R.k0, ty) > b.L.partials_cap)
                 ty *= 2;
-            int streams = first ? (fu ? 4 : 3) : 5;     // reads
+            int streams = (first ? (fu ? 2 : 1) : 3) + kstreams(c, b);  // reads
             streams += (fu ? 1 : 0) + (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})
             const int kid = last ? TEA_K_TB_LAST : (first ? TEA_K_TB_FIRST : TEA_K_TB_MID);
             K(c, kid, sbytes(b, streams), [&] {
@@ -692,7 +700,7 @@ void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan_spmv(c, b, R);
-        K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
+        K(c, TEA_K_SPMV, sbytes(b, 6 + kstreams(c, b)), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[zs], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
         });
@@ -717,7 +725,7 @@ void body_bj(tea_ctx *c, int par, bool sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan_spmv(c, b, R);
-        K(c, TEA_K_SPMV, sbytes(b, 8), [&] {
+        K(c, TEA_K_SPMV, sbytes(b, 6 + kstreams(c, b)), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[F_Z0], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
         });
@@ -1251,6 +1259,7 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
         if (o.loop_mode < 0 || o.loop_mode > 2) fail(TEA_ERR_ARG, "bad loop_mode");
         if (o.persist < -1 || o.persist > 1) fail(TEA_ERR_ARG, "bad persist");
         if (o.overlap < -1 || o.overlap > 1) fail(TEA_ERR_ARG, "bad overlap");
+        if (o.kform < -1 || o.kform > 1) fail(TEA_ERR_ARG, "bad kform");
         // NCCL kernels inside a WHILE-conditional graph body are not a supported
         // capture target: multi-process runs use chunked graphs (same kernels).
         if (nranks > 1 && o.loop_mode == 0) o.loop_mode = 1;
@@ -1345,10 +1354,13 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
             Region all{-d, L.bx + d + 1, -d, L.by + d + 1};
             Region kxr{-d, L.bx + d + 1, -d, L.by + d};
             Region kyr{-d, L.bx + d, -d, L.by + d + 1};
+            // g on every cell a face of kxr / kyr touches; the stored
+            // faces are formed from the same g by the same expression as the kernels'
+            Region gall{-d - 1, L.bx + d + 1, -d - 1, L.by + d + 1};
             K(c.get(), TEA_K_INIT, 0.0, [&] {
                 launch_init_fields(kargs(c.get(), b), b.f[F_W], b.f[F_Z0], b.f[F_U0], b.f[F_U],
-                                   b.f[F_KX], b.f[F_KY], owned, all, kxr, kyr, c->rx, c->ry,
-                                   o.mean_mode, c->stream);
+                                   b.f[F_KX], b.f[F_KY], b.f[F_KZ], owned, all, kxr, kyr, gall,
+                                   0.5 * c->rx, 0.5 * c->ry, o.mean_mode, c->stream);
             });
             K(c.get(), TEA_K_INIT, 0.0, [&] {
                 launch_bj_setup(kargs(c.get(), b), owned, b.f[F_KX], b.f[F_KY], b.f[F_BJC],

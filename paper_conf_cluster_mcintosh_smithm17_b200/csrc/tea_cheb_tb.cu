@@ -281,7 +281,11 @@ struct TbGeom {
 #endif
 constexpr int kTmCols = 128;  // TMEM columns per 4 warps: 8 slots x 16 per warp quarter
 
-template <int M, bool FIRST, bool FUSE, bool LAST>
+// KG (tea_opts.kform): Kx points at g = 1/rho and the row's faces are formed
+// as it arrives -- Kx(j) = hrx (g(j-1) + g(j)) with g(j-1) from the west lane (lane 0's
+// west face is a margin column, polluted like its west operand), Ky(k) = hry (g(k-1) + g(k))
+// with g(k-1) the previous row's -- one staged stream instead of two, same faces bit for bit.
+template <int M, bool FIRST, bool FUSE, bool LAST, bool KG>
 __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     k_cheb_tb(const double *__restrict__ rin, const double *__restrict__ win,
               double *__restrict__ rout, const double *__restrict__ zin1,
@@ -381,7 +385,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                 cp16(&cpa[sl][2][threadIdx.x], rin + o);
             }
             cp16(&cpa[sl][3][threadIdx.x], Kx + o);
-            cp16(&cpa[sl][4][threadIdx.x], Ky + o);
+            if (!KG) cp16(&cpa[sl][4][threadIdx.x], Ky + o);
         }
         cp_commit();  // one group per row, empty or not, so wait_group counts rows
     };
@@ -395,12 +399,27 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     int cs = 0;    // staging slot of row k
     int head = 0;  // TMEM ring slot of row k
     double2 z2prev = z0;  // z_{i-2} input of the previous row (a one-row register delay)
+    double2 gprev = z0;   // KG: g of the previous input row (row kbeg-1's only feeds the
+                          // pipeline-fill rows every pass discards)
+    const double hrx = a.hrx, hry = a.hry;
     constexpr int UNR = FIRST ? kTbUnroll : kTbUnrollL;
 #pragma unroll(UNR)
     for (int k = kbeg; k < kend; ++k, orow += pitch, head = (head + 1) & (D - 1)) {
         cp_wait<P - 1>();  // row k's group (the oldest outstanding) has landed
         double2 X = cpa[cs][0][threadIdx.x];
-        const double2 KX = cpa[cs][3][threadIdx.x], KY = cpa[cs][4][threadIdx.x];
+        double2 KX, KY;
+        if (KG) {
+            const double2 g = cpa[cs][3][threadIdx.x];
+            const double gW = __shfl_up_sync(0xffffffffu, g.y, 1);
+            KX.x = hrx * (gW + g.x);
+            KX.y = hrx * (g.x + g.y);
+            KY.x = hry * (gprev.x + g.x);
+            KY.y = hry * (gprev.y + g.y);
+            gprev = g;
+        } else {
+            KX = cpa[cs][3][threadIdx.x];
+            KY = cpa[cs][4][threadIdx.x];
+        }
         double2 Wv = z0, Z2 = z0, RR = z0;
         if (FIRST) {
             if (FUSE) Wv = cpa[cs][1][threadIdx.x];
@@ -580,7 +599,7 @@ int tb_out_cols(int M) {
     return kStrip - 2 * mr;
 }
 
-template <int M, bool FIRST, bool FUSE, bool LAST>
+template <int M, bool FIRST, bool FUSE, bool LAST, bool KG>
 static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty, int jlim,
                       int step0, bool restart,
                       const double *rin, const double *win, double *rout, const double *zin1,
@@ -593,11 +612,11 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
     constexpr size_t smem = tb_smem_bytes();
     static bool attr = false;  // per instantiation
     if (!attr) {
-        cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST>,
+        cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST, KG>,
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         attr = true;
     }
-    k_cheb_tb<M, FIRST, FUSE, LAST><<<grid, kTbT, smem, st>>>(
+    k_cheb_tb<M, FIRST, FUSE, LAST, KG><<<grid, kTbT, smem, st>>>(
         rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, a, R, Dd, ty, jlim, step0, restart ? 1 : 0);
 }
 
@@ -608,8 +627,14 @@ static void tb_dispatch(const KArgs &a, const Region &R, const Region &Dd, int t
                         double *rout, const double *zin1, const double *zin2, double *zoutA,
                         double *zoutB, const double *kx, const double *ky, cudaStream_t st) {
 #define TB(F, U, L)                                                                            \
-    tb_launch<M, F, U, L>(a, R, Dd, ty, jlim, step0, restart, rin, win, rout, zin1, zin2, zoutA, \
-                          zoutB, kx, ky, st)
+    do {                                                                                       \
+        if (a.g)                                                                               \
+            tb_launch<M, F, U, L, true>(a, R, Dd, ty, jlim, step0, restart, rin, win, rout, zin1, \
+                                        zin2, zoutA, zoutB, a.g, nullptr, st);                 \
+        else                                                                                   \
+            tb_launch<M, F, U, L, false>(a, R, Dd, ty, jlim, step0, restart, rin, win, rout,     \
+                                         zin1, zin2, zoutA, zoutB, kx, ky, st);                \
+    } while (0)
     if (first) {
         if (fuse) {
             if (last) TB(true, true, true); else TB(true, true, false);
@@ -639,9 +664,10 @@ int tb_auto_rows(int M, int width, int height) {
         switch (M) {
 #define OCC(m)                                                                                   \
     case m:                                                                                      \
-        cudaFuncSetAttribute(k_cheb_tb<m, false, false, true>,                                   \
+        cudaFuncSetAttribute(k_cheb_tb<m, false, false, true, true>,                             \
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);            \
-        e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per, k_cheb_tb<m, false, false, true>, \
+        e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per,                                  \
+                                                          k_cheb_tb<m, false, false, true, true>, \
                                                           kTbT, smem);                       \
         break;
             OCC(1) OCC(2) OCC(3) OCC(4) OCC(5)

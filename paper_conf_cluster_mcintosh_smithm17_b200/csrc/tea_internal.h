@@ -83,6 +83,12 @@ struct KArgs {
     long long ps;
     int nz;
     int coef_slot;  // constant-memory coefficient slot of the fused passes (tea_cheb_tb.cu)
+    // 2D on-the-fly faces (tea_opts.kform): g = 1/rho (or rho) on the block
+    // plus margin, ghost cells outside the mesh hold -g of their interior neighbour so the
+    // physical-boundary faces come out exactly 0; Kx(j,k) = hrx (g(j-1,k) + g(j,k)),
+    // Ky(j,k) = hry (g(j,k-1) + g(j,k)). g == nullptr: the kernels read the stored Kx, Ky.
+    const double *g;
+    double hrx, hry;
 };
 
 Launch plan_stencil(const Region &R, int ty_req, int ncta_target);
@@ -95,9 +101,9 @@ Launch plan_pointwise(const Region &R, int ty_req, int ncta_target);
 int max_ctas(int width, int height);
 
 void launch_init_fields(const KArgs &a, const double *rho, const double *en, double *u0,
-                        double *u, double *kx, double *ky, Region owned, Region all,
-                        Region kxr, Region kyr, double rx, double ry, int mean_mode,
-                        cudaStream_t st);
+                        double *u, double *kx, double *ky, double *g, Region owned, Region all,
+                        Region kxr, Region kyr, Region gall, double hrx, double hry,
+                        int mean_mode, cudaStream_t st);
 // 3D: Kx, Ky, Kz (rz = dt/dz^2) and u0 = u = rho e on the single block (planes [0, nz))
 void launch_init_fields3(const KArgs &a, const double *rho, const double *en, double *u0,
                          double *u, double *kx, double *ky, double *kz, int nx, int ny, int nz,

@@ -667,3 +667,43 @@ def test_persist_many_tiles_per_cta(tea, tile_rows):
     assert st_p[0]["iterations"] == st_g[0]["iterations"] == 33
     assert st_p[0]["outer"] == st_g[0]["outer"] == 3
     assert rel_err(u_p, u_g) <= 1e-12
+
+
+# ---------------------------------------------------------------- kform
+@pytest.mark.gpu
+@pytest.mark.parametrize("kind,nx,ny", [("pipe", 128, 128), ("random", 300, 200),
+                                        ("random", 1000, 777), ("random", 257, 65),
+                                        ("random", 1, 97), ("random", 95, 1)])
+@pytest.mark.parametrize("method,tb", [(0, 0), (1, 5), (1, 1), (1, 3), (2, 0), (3, 0), (6, 5)])
+@pytest.mark.parametrize("mean_mode", [0, 1])
+def test_kform_bitwise(tea, kind, nx, ny, method, tb, mean_mode):
+    """Faces formed on the fly from g = 1/rho (kform 1) and read as the stored Kx, Ky
+    (kform -1) are the same numbers (the stored faces are computed by the kernels'
+    expression), so the whole solve is bitwise identical: fixed iterations and converged."""
+    deck = deck_of(kind, nx, ny, seed=5, dt=0.04)
+    for eps, its in ((0.0, 37), (1e-13, 20000)):
+        kw = dict(method=method, eps=eps, max_iters=its, inner_steps=6, tb_steps=tb,
+                  persist=-1, mean_mode=mean_mode)
+        u_g, st_g = gpu_run(tea, deck, kform=1, **dict(kw))
+        u_k, st_k = gpu_run(tea, deck, kform=-1, **dict(kw))
+        assert st_g[0]["iterations"] == st_k[0]["iterations"]
+        assert np.array_equal(u_g, u_k)
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("blocks,d", [((2, 2), 1), ((2, 2), 7), ((3, 2), 4)])
+@pytest.mark.parametrize("method", [0, 1, 6])
+def test_kform_bitwise_blocks(tea, ora, blocks, d, method):
+    """Decomposed (blocks in one process, halo depth d): g carries real neighbour values in
+    the margin and mirrored ghosts at the physical boundary -- bitwise equal to the stored
+    faces, and within the parity bar of the oracle."""
+    deck = deck_of("random", 301, 203, seed=6, dt=0.04)
+    dist = dict(rank=0, nranks=1, px=blocks[0], py=blocks[1], halo_depth=d)
+    kw = dict(method=method, eps=1e-13, max_iters=20000, inner_steps=6)
+    u_g, st_g = gpu_run(tea, deck, dist=dist, kform=1, **dict(kw))
+    u_k, st_k = gpu_run(tea, deck, dist=dist, kform=-1, **dict(kw))
+    assert st_g[0]["iterations"] == st_k[0]["iterations"]
+    assert np.array_equal(u_g, u_k)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert field_err(u_g, u_o, "random") <= 1e-10
