@@ -204,7 +204,8 @@ def config(args):
             "mesh": [args.n, args.n] + ([args.nz] if args.nz > 1 else []),
             "method": args.method, "inner_steps": args.inner,
             "eps": args.eps, "max_iters": args.max_iters, "halo_depth": args.halo_depth,
-            "dt": 0.004, "kform": "stored Kx, Ky" if args.kform < 0 else "g = 1/rho on the fly",
+            "dt": 0.004, "kform": ("stored Kx, Ky, Kz (3D)" if args.nz > 1 else
+                                    "stored Kx, Ky" if args.kform < 0 else "g = 1/rho on the fly"),
             "l2": "inputs larger than L2 (>= 12 fp64 fields x 8 B x cells > 126 MB)"
             if args.n * args.n * max(args.nz, 1) >= 2 ** 21 else
             "working set fits in L2 (no flush)"}

@@ -532,7 +532,8 @@ int cheb_chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, b
                 const double *z1 = step >= 2 ? b.f[zbuf(step - 1)] : nullptr;
                 const double *z2 = step >= 3 ? b.f[zbuf(step - 2)] : nullptr;
                 int kid = step == 1 ? TEA_K_CHEB_FIRST : (last ? TEA_K_CHEB_LAST : TEA_K_CHEB_STEP);
-                const int streams = mode == 0 ? (fu ? 6 : 4) : (mode == 1 ? 5 : 6);
+                const int streams =
+                    (mode == 0 ? (fu ? 4 : 2) : (mode == 1 ? 3 : 4)) + kstreams(c, b);
                 K(c, kid, sbytes(b, streams), [&] {
                     launch_cheb(kargs(c, b, last && sets_cond), L, R, D, mode, step, last, fu,
                                 restart, b.f[fu ? rin : r], b.f[F_W], b.f[rout], z1, z2,
@@ -750,7 +751,7 @@ void body_cg1(tea_ctx *c, int par, bool sets_cond) {
         BlockCtx &b = c->blocks[0];
         Region R = b.owned();
         Launch L = plan_st(c, b, R);
-        K(c, TEA_K_CG1, sbytes(b, 12), [&] {
+        K(c, TEA_K_CG1, sbytes(b, 10 + kstreams(c, b)), [&] {
             launch_cg1(kargs(c, b, sets_cond), L, R, b.f[F_R0 + par], b.f[F_Z0 + par],
                        b.f[F_Z2 + par], b.f[F_R1 - par], b.f[F_Z1 - par], b.f[F_Z3 - par],
                        b.f[F_P0], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
@@ -769,7 +770,7 @@ void body_cg1(tea_ctx *c, int par, bool sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan_st(c, b, R);
-        K(c, TEA_K_CG1W, sbytes(b, 4), [&] {
+        K(c, TEA_K_CG1W, sbytes(b, 2 + kstreams(c, b)), [&] {
             launch_cg1_w(kargs(c, b, sets_cond), L, R, b.f[F_R0], b.f[F_Z0], b.f[F_KX],
                          b.f[F_KY], c->stream);
         });
@@ -796,7 +797,7 @@ void body_pcg1(tea_ctx *c, int s, int /*par*/, bool sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan_st(c, b, R);
-        K(c, TEA_K_CG1W, sbytes(b, 4), [&] {
+        K(c, TEA_K_CG1W, sbytes(b, 2 + kstreams(c, b)), [&] {
             launch_cg1_w(kargs(c, b, sets_cond), L, R, b.f[zs], b.f[F_W], b.f[F_KX], b.f[F_KY],
                          c->stream, true);
         });
@@ -811,7 +812,7 @@ void body_stat(tea_ctx *c, bool cheb, int par, bool sets_cond) {
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan_st(c, b, R);
-        K(c, TEA_K_STAT, sbytes(b, cheb ? 6 : 5), [&] {
+        K(c, TEA_K_STAT, sbytes(b, (cheb ? 4 : 3) + kstreams(c, b)), [&] {
             launch_stat(kargs(c, b, sets_cond), L, R, cheb, b.f[in], b.f[F_U0], b.f[out],
                         b.f[F_KX], b.f[F_KY], c->stream);
         });
@@ -1007,7 +1008,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan_st(c, b, R);
-        K(c, TEA_K_RESIDUAL, sbytes(b, 5), [&] {
+        K(c, TEA_K_RESIDUAL, sbytes(b, 3 + kstreams(c, b)), [&] {
             launch_residual(kargs(c, b), L, R, b.f[F_U], b.f[F_KX], b.f[F_KY], b.f[F_U0],
                             b.f[F_R0], c->stream);
         });
@@ -1026,7 +1027,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         for (auto &b : c->blocks) {
             Region R = b.owned();
             Launch L = plan_st(c, b, R);
-            K(c, TEA_K_CG1W, sbytes(b, 4), [&] {
+            K(c, TEA_K_CG1W, sbytes(b, 2 + kstreams(c, b)), [&] {
                 launch_cg1_w(kargs(c, b), L, R, b.f[F_R0], b.f[F_Z0], b.f[F_KX], b.f[F_KY],
                              c->stream);
             });
@@ -1088,7 +1089,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
             for (auto &b : c->blocks) {
                 Region R = b.owned();
                 Launch L = plan_st(c, b, R);
-                K(c, TEA_K_CG1W, sbytes(b, 4), [&] {
+                K(c, TEA_K_CG1W, sbytes(b, 2 + kstreams(c, b)), [&] {
                     launch_cg1_w(kargs(c, b), L, R, b.f[zs], b.f[F_W], b.f[F_KX], b.f[F_KY],
                                  c->stream, true);
                 });

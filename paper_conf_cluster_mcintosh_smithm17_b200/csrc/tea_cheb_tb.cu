@@ -411,10 +411,12 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         if (KG) {
             const double2 g = cpa[cs][3][threadIdx.x];
             const double gW = __shfl_up_sync(0xffffffffu, g.y, 1);
-            KX.x = hrx * (gW + g.x);
-            KX.y = hrx * (g.x + g.y);
-            KY.x = hry * (gprev.x + g.x);
-            KY.y = hry * (gprev.y + g.y);
+            // __dmul_rn: never contracted into an FMA with the faces' uses (the diagonal
+            // sum below), so every face equals the stored one bit for bit
+            KX.x = __dmul_rn(hrx, gW + g.x);
+            KX.y = __dmul_rn(hrx, g.x + g.y);
+            KY.x = __dmul_rn(hry, gprev.x + g.x);
+            KY.y = __dmul_rn(hry, gprev.y + g.y);
             gprev = g;
         } else {
             KX = cpa[cs][3][threadIdx.x];

@@ -674,16 +674,21 @@ def test_persist_many_tiles_per_cta(tea, tile_rows):
 @pytest.mark.parametrize("kind,nx,ny", [("pipe", 128, 128), ("random", 300, 200),
                                         ("random", 1000, 777), ("random", 257, 65),
                                         ("random", 1, 97), ("random", 95, 1)])
-@pytest.mark.parametrize("method,tb", [(0, 0), (1, 5), (1, 1), (1, 3), (2, 0), (3, 0), (6, 5)])
+@pytest.mark.parametrize("method,tb,persist", [(0, 0, -1), (1, 5, -1), (1, 1, -1), (1, 3, -1),
+                                               (2, 0, -1), (3, 0, -1), (6, 5, -1), (6, 1, -1),
+                                               (0, 0, 1), (1, 1, 1), (4, 0, -1), (5, 0, -1)])
 @pytest.mark.parametrize("mean_mode", [0, 1])
-def test_kform_bitwise(tea, kind, nx, ny, method, tb, mean_mode):
+def test_kform_bitwise(tea, kind, nx, ny, method, tb, persist, mean_mode):
     """Faces formed on the fly from g = 1/rho (kform 1) and read as the stored Kx, Ky
     (kform -1) are the same numbers (the stored faces are computed by the kernels'
-    expression), so the whole solve is bitwise identical: fixed iterations and converged."""
-    deck = deck_of(kind, nx, ny, seed=5, dt=0.04)
-    for eps, its in ((0.0, 37), (1e-13, 20000)):
+    expression), so the whole solve is bitwise identical: fixed iterations and converged,
+    for every 2D stencil kernel (SpMV, fused passes, per-step Chebyshev, CG1 / CPPCG1,
+    block Jacobi, the persistent solver, Jacobi / Chebyshev iterations)."""
+    stationary = method in (4, 5)
+    deck = deck_of(kind, nx, ny, seed=5, dt=0.004 if stationary else 0.04)
+    for eps, its in ((0.0, 37), (1e-13, 3000 if stationary else 20000)):
         kw = dict(method=method, eps=eps, max_iters=its, inner_steps=6, tb_steps=tb,
-                  persist=-1, mean_mode=mean_mode)
+                  persist=persist, mean_mode=mean_mode, presteps=10 if stationary else 30)
         u_g, st_g = gpu_run(tea, deck, kform=1, **dict(kw))
         u_k, st_k = gpu_run(tea, deck, kform=-1, **dict(kw))
         assert st_g[0]["iterations"] == st_k[0]["iterations"]

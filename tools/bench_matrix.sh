@@ -5,6 +5,7 @@ OUT=${1:-gpurun_out/bench_matrix.jsonl}
 : > $OUT
 run() { timeout 600 python bench.py "$@" --no-cpu 2>/dev/null | tail -1 >> $OUT; }
 run --method cppcg --n 4096 --steps 5 --warmup 3
+run --method cppcg --n 4096 --steps 5 --warmup 3 --kform -1   # stored faces (A/B, §4.13)
 run --method cg --n 4096 --steps 3 --warmup 3
 run --method cg1 --n 4096 --steps 3 --warmup 3
 run --method bjcg --n 4096 --steps 3 --warmup 3
@@ -29,7 +30,8 @@ for l in open(sys.argv[1]):
     try: d = json.loads(l)
     except Exception: continue
     r = d["roofline"]
-    print(f"{d['config']['workload'] + ' ' + d['config']['parallelism']:62s} {d['value']:9.1f} it/s  {d['time_to_solution_s']*1e3:9.2f} ms/step "
+    kf = '' if d['config'].get('kform', 'g').startswith('g') else ' [stored K]'
+    print(f"{d['config']['workload'] + ' ' + d['config']['parallelism'] + kf:62s} {d['value']:9.1f} it/s  {d['time_to_solution_s']*1e3:9.2f} ms/step "
           f"its={d['iterations_per_step']:.0f} model={d['hbm_gbs_model']:.0f}GB/s dom={r['kernel']} "
           f"frac={r['frac']:.3f}")
 PY

@@ -94,6 +94,7 @@ def main():
         subprocess.call(["cp", ll, os.path.join(prof, f"{tag}_launches_bench{n}.csv")])
     # traffic per launch for bench.py: average over the captured launches of each class
     key = {"k_cheb_tb<5, 1, 1, 0>": "tb_first", "k_cheb_tb<5, 0, 0, 1>": "tb_last",
+           "k_cheb_tb<5, 1, 1, 0, 1>": "tb_first", "k_cheb_tb<5, 0, 0, 1, 1>": "tb_last",
            "k_spmv<0>": "spmv", "k_spmv": "spmv"}
     tp = os.path.join(prof, "ncu_traffic.json")
     traffic = json.load(open(tp))
@@ -105,6 +106,8 @@ def main():
     for cls, v in per.items():
         ent = traffic.setdefault(f"{cls}@{n}", {})
         ent["dram_bytes_per_launch"] = int(sum(x for x, _ in v) / len(v))
+        # algorithmic bytes of the form profiled (faces from g: DESIGN.md §4.13)
+        ent["algorithmic_bytes_per_launch"] = {"spmv": 7, "tb_first": 6, "tb_last": 5}[cls] * 8 * n * n
         ent["kernel"] = v[0][1]
         ent["round"] = tag[1:] if tag.startswith("r") else tag
     json.dump(traffic, open(tp, "w"), indent=1)
