@@ -253,6 +253,14 @@ Launch plan_st(tea_ctx *c, const BlockCtx &b, const Region &R) {
 // the SpMV: large 2D blocks (where the default tile is the 32-row cap) get wave-fitted tiles
 Launch plan_spmv(tea_ctx *c, const BlockCtx &b, const Region &R) {
     Launch L = plan_st(c, b, R);
+    if (b.L.nz > 1 && c->opts.tile_rows <= 0) {
+        // 3D: one wave at the SpMV's 4 CTAs/SM (TEA_SPMV3_MINB), so each warp marches as many
+        // planes as fit -- fewer (tz + 2) / tz re-read planes (256^3: tz 32 -> 128, SpMV
+        // 4776 -> 4965 GB/s, profiles/r01k_tz3.txt)
+        const int cols = (int)(L.grid.x * L.grid.y);
+        const int gz = std::max(1, 592 / std::max(cols, 1));
+        return plan_stencil3(R, b.L.nz, std::max(4, (b.L.nz + gz - 1) / gz));
+    }
     if (b.L.nz > 1 || c->opts.tile_rows > 0 || c->ty_override > 0 || L.ty < 32) return L;
     const int ty = spmv_wave_rows(R.j1 - L.jstart, R.k1 - R.k0);
     // one reduction partial per CTA must fit the block's scratch (fewer CTAs: always true)
