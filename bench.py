@@ -11,12 +11,19 @@ value       solver iterations/s (CG presteps + CPPCG outer iterations, tea_stats
 e2e         same metric through the C ABI with HOST buffers: each step copies
             u^n host->device (tea_set_u, pinned), solves, copies u^{n+1} back
             (tea_fetch) inside the timed region.
-roofline    the dominant kernel (the Chebyshev inner step):
-            algorithmic bytes per launch / its mean launch duration from a
-            profiled solve (CUDA events around each launch on the library's
-            stream); peak = MEASURED_PEAKS.json hbm_gbs.
-cpu_baseline the CPU oracle (oracle/, serial C, 1 thread) on a bounded prefix of
-            the same timestep, same unit.
+roofline    the dominant kernel = the kernel class with the largest share of the
+            timed region's device time: algorithmic bytes per launch (DESIGN.md
+            §4 model) / its mean launch duration, both taken INSIDE the timed
+            WHILE-graph solves by the library's in-graph timing (tea_opts.trace:
+            %globaltimer at each launch's start and at its last CTA's end;
+            no-op launches after convergence and the finalising u update are
+            not counted); peak = MEASURED_PEAKS.json hbm_gbs; traffic = ncu
+            DRAM bytes per launch from profiles/ncu_traffic.json, used only when
+            its recorded source hash matches the built library's sources.
+cpu_baseline the CPU oracle (oracle/, serial C, 1 thread) timed on bounded
+            samples of the same timestep (30 presteps; + the restart and 1 outer
+            iteration; + 1 more outer iteration), its per-phase costs weighted by
+            the GPU run's own iteration mix (like for like), and matvecs/s.
 
 Usage: python bench.py [--gpus N] [--steps K] [--warmup W] [--impl reference]
        [--n 4096] [--method cppcg|cg] [--inner 10] [--eps 1e-12] [--halo-depth d]
@@ -123,52 +130,166 @@ def cg_iter_bytes(cells):
     return 11 * 8 * cells
 
 
+def source_hash():
+    """sha256 (16 hex) of the CUDA library's sources: stamps ncu-derived numbers."""
+    import hashlib
+    h = hashlib.sha256()
+    base = os.path.join(ROOT, "paper_conf_cluster_mcintosh_smithm17_b200", "csrc")
+    for f in sorted(os.listdir(base)) + ["../../include/tea.h"]:
+        if f.endswith((".cu", ".h")):
+            h.update(open(os.path.join(base, f), "rb").read())
+    return h.hexdigest()[:16]
+
+
 def load_ncu_traffic(kernel_key, n):
+    """ncu DRAM bytes per launch of kernel class `kernel_key` at mesh n, if captured from
+    the current sources (profiles/ncu_traffic.json entries carry the source hash)."""
     p = os.path.join(ROOT, "profiles", "ncu_traffic.json")
     if not os.path.exists(p):
-        return None
-    d = json.load(open(p))
-    e = d.get(f"{kernel_key}@{n}")
-    return None if e is None else float(e["dram_bytes_per_launch"])
+        return None, "no profiles/ncu_traffic.json"
+    e = json.load(open(p)).get(f"{kernel_key}@{n}")
+    if e is None:
+        return None, f"no capture of {kernel_key}@{n}"
+    if e.get("source_hash") != source_hash():
+        return None, f"capture of {kernel_key}@{n} is from other sources ({e.get('source_hash')})"
+    return float(e["dram_bytes_per_launch"]), f"profiles/ncu_traffic.json ({e.get('capture')})"
+
+
+def cpu_info():
+    info = {}
+    try:
+        for line in open("/proc/cpuinfo"):
+            k, _, v = line.partition(":")
+            k = k.strip()
+            if k in ("model name", "cpu family", "model") and k not in info:
+                info[k] = v.strip()
+            if len(info) == 3:
+                break
+    except OSError:
+        pass
+    return {"cpu_model": f"{info.get('model name', 'unknown')} (family {info.get('cpu family', '?')}"
+                         f" model {info.get('model', '?')})",
+            "host_cores_available": len(os.sched_getaffinity(0)), "oracle_threads": 1}
+
+
+# ------------------------------------------------------------------ oracle timing
+TWO_PHASE = ("cppcg", "cppcg1", "cheby")
+# iteration mix of one timestep of the headline workload on the GPU (4096^2 pipe CPPCG s=10,
+# eps 1e-12, timesteps 6-25 of the bench: 30 presteps + 253.1 outer, profiles/r01j_bench.json;
+# the oracle's counts agree within +-2, tests/test_gpu_parity.py): used by the reference arm,
+# which cannot run the GPU, to weight its per-phase costs like the GPU arm's cpu_baseline
+HEADLINE_MIX = (30.0, 253.1)
+
+
+def oracle_phase_costs(args, deck):
+    """Serial oracle costs of the phases of one timestep, measured on bounded samples:
+    two-phase methods run 30 presteps, then 30 + restart + 1 outer, then + 1 more outer
+    (t_pre per prestep, t_restart = eigen-estimate + restart chain, t_outer per outer);
+    one-phase methods run 20 iterations. Solve time only (faces precomputed)."""
+    import oracle
+    oracle.build()
+    method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
+              "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY,
+              "cppcg1": oracle.CPPCG1}[args.method]
+    if args.nz > 1:
+        rx, ry, rz = oracle.mesh_r3(deck)
+        K = oracle.face_coefficients3(deck.nx, deck.ny, deck.nz, rx, ry, rz, deck.density)
+
+        def solve(its):
+            return oracle.solve3(*K, deck.density * deck.energy, None, method, args.eps, its,
+                                 args.inner)
+    else:
+        rx, ry = oracle.mesh_r(deck)
+        K = oracle.face_coefficients(deck.nx, deck.ny, rx, ry, deck.density)
+
+        def solve(its):
+            return oracle.solve(*K, deck.density * deck.energy, None, method, args.eps, its,
+                                args.inner)
+
+    def timed(its):
+        t0 = time.perf_counter()
+        r = solve(its)
+        return time.perf_counter() - t0, r.stats
+
+    if args.method in TWO_PHASE:
+        t30, s30 = timed(30)
+        t31, s31 = timed(31)
+        t32, s32 = timed(32)
+        t_outer = t32 - t31
+        c = {"t_pre": t30 / 30, "t_restart": max(t31 - t30 - t_outer, 0.0), "t_outer": t_outer,
+             "sample_s": t30 + t31 + t32, "matvecs_per_s": (s30["matvecs"] + s31["matvecs"] +
+                                                          s32["matvecs"]) / (t30 + t31 + t32),
+             "sample": "30 presteps; 30 presteps + restart + 1 outer; + 1 more outer"}
+    else:
+        t20, s20 = timed(20)
+        c = {"t_it": t20 / 20, "sample_s": t20, "matvecs_per_s": s20["matvecs"] / t20,
+             "sample": "20 iterations"}
+    return c
+
+
+def cpu_time_for_mix(c, presteps, outer, iters):
+    """Oracle seconds for one timestep with the given iteration mix (per-phase costs)."""
+    if "t_pre" in c:
+        return presteps * c["t_pre"] + (c["t_restart"] if outer > 0 else 0.0) + outer * c["t_outer"]
+    return iters * c["t_it"]
 
 
 # ------------------------------------------------------------------ reference arm
 def run_reference(args):
-    import oracle
-    from paper_conf_cluster_mcintosh_smithm17_b200 import inputs
-
+    """The reference arm for this tier: the CPU oracle as it stands, 1 thread, on the same
+    workload. Warm-up 1 measures its per-phase costs (oracle_phase_costs); each timed step
+    re-times the 31-iteration sample (30 presteps + restart + 1 outer) and is charged the
+    CPU time of a full timestep of the headline's iteration mix scaled by it."""
     rank = int(os.environ.get("RANK", "0"))
     if rank != 0:
         return 0
+    import oracle
     oracle.build()
     deck = make_deck(args)
     method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
               "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY,
               "cppcg1": oracle.CPPCG1}[args.method]
-    sample_iters = args.ref_iters
     orun = oracle.run3 if args.nz > 1 else oracle.run
-    for _ in range(args.warmup):  # untimed warm-up (page-in, caches)
-        orun(deck, steps=1, method=method, eps=args.eps, max_iters=1, inner_steps=args.inner)
-    t_all, its, mv = 0.0, 0, 0
+    costs = oracle_phase_costs(args, deck)  # (part of the warm-up)
+    two = "t_pre" in costs
+    mix = (HEADLINE_MIX if (args.method == "cppcg" and args.n == 4096 and args.inner == 10
+                            and args.nz <= 1) else None)
+    sample_iters = 31 if two else 20
+    t_sample_warm = None
+    for _ in range(max(args.warmup - 1, 1)):
+        t0 = time.perf_counter()
+        orun(deck, steps=1, method=method, eps=args.eps, max_iters=sample_iters,
+             inner_steps=args.inner)
+        t_sample_warm = time.perf_counter() - t0
+    t_all, t_charged, its, mv = 0.0, 0.0, 0.0, 0
     for _ in range(args.steps):
         t0 = time.perf_counter()
         _, st, _ = orun(deck, steps=1, method=method, eps=args.eps, max_iters=sample_iters,
                         inner_steps=args.inner)
-        t_all += time.perf_counter() - t0
-        its += st[0]["iterations"]
+        dt = time.perf_counter() - t0
+        t_all += dt
         mv += st[0]["matvecs"]
-    value = its / t_all
-    sample = (f"first {sample_iters} iterations of timestep 1 ("
-              + (f"30 CG presteps + {sample_iters - 30} CPPCG outer" if args.method == "cppcg"
-                 else METHOD_NAME[args.method]) + ") per step, serial C oracle")
+        if mix is not None:
+            t_charged += cpu_time_for_mix(costs, mix[0], mix[1], 0) * dt / t_sample_warm
+            its += mix[0] + mix[1]
+        else:
+            t_charged += dt
+            its += st[0]["iterations"]
+    value = its / t_charged
+    sample = (f"{sample_iters} iterations of timestep 1 per step (serial C oracle, 1 thread)"
+              + (f", charged as a full timestep of the GPU's iteration mix ({mix[0]:g} presteps"
+                 f" + {mix[1]:g} outer) from the oracle's per-phase costs ({costs['sample']}:"
+                 f" {costs['t_pre']:.3f} s/prestep, restart {costs['t_restart']:.2f} s,"
+                 f" {costs['t_outer']:.2f} s/outer)" if mix else ""))
     line = {
         "impl": "reference", "metric": metric_name(args), "value": value, "unit": "iterations/s",
         "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
         "ms_per_step": 1e3 * t_all / args.steps, "higher_is_better": True,
         "scaling": "strong", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
         "config": config(args),
-        "cpu_baseline": {"value": value, "unit": "iterations/s", "cores": 1, "kind": "oracle",
-                         "sample": sample, "matvecs_per_s": mv / t_all},
+        "cpu_baseline": dict({"value": value, "unit": "iterations/s", "cores": 1,
+                              "kind": "oracle", "sample": sample,
+                              "matvecs_per_s": mv / t_all}, **cpu_info()),
         "e2e": {"value": value, "unit": "iterations/s", "h2d_bytes_per_step": 0,
                 "d2h_bytes_per_step": 0},
     }
@@ -212,24 +333,24 @@ def config(args):
 
 
 # ------------------------------------------------------------------ GPU arm
-def cpu_baseline(args, deck):
-    import oracle
-    oracle.build()
-    method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
-              "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY,
-              "cppcg1": oracle.CPPCG1}[args.method]
-    t0 = time.perf_counter()
-    orun = oracle.run3 if args.nz > 1 else oracle.run
-    _, st, _ = orun(deck, steps=1, method=method, eps=args.eps, max_iters=args.ref_iters,
-                    inner_steps=args.inner)
-    dt = time.perf_counter() - t0
-    return {"value": st[0]["iterations"] / dt, "unit": "iterations/s", "cores": 1,
-            "kind": "oracle",
-            "sample": f"first {args.ref_iters} iterations of timestep 1 ("
-                      + (f"{st[0]['presteps']} CG presteps + {st[0]['outer']} CPPCG outer"
-                         if args.method == "cppcg" else METHOD_NAME[args.method])
-                      + f"), serial C oracle, {dt:.1f} s",
-            "matvecs_per_s": st[0]["matvecs"] / dt}
+def cpu_baseline(args, deck, stats):
+    """The oracle (1 thread) like for like: its measured per-phase costs weighted by this
+    run's own iteration mix (presteps / outer iterations per timestep, averaged)."""
+    c = oracle_phase_costs(args, deck)
+    k = len(stats)
+    pre = sum(s["presteps"] for s in stats) / k
+    outer = sum(s["outer"] for s in stats) / k
+    iters = sum(s["iterations"] for s in stats) / k
+    t_step = cpu_time_for_mix(c, pre, outer, iters)
+    mix = (f"{pre:g} presteps + {outer:g} outer" if "t_pre" in c else f"{iters:g} iterations")
+    return dict({"value": iters / t_step, "unit": "iterations/s", "cores": 1, "kind": "oracle",
+                 "sample": f"serial C oracle timed on {c['sample']} of timestep 1 "
+                           f"({c['sample_s']:.1f} s); per-phase costs weighted by this run's "
+                           f"mix per timestep ({mix}): {t_step:.1f} s per timestep "
+                           "(extrapolated)",
+                 "matvecs_per_s": c["matvecs_per_s"],
+                 "phase_costs_s": {k2: round(v, 4) for k2, v in c.items()
+                                   if k2.startswith("t_")}}, **cpu_info())
 
 
 def factor(n):
@@ -291,7 +412,8 @@ def run_gpu(args):
     cells = args.n * args.n * max(args.nz, 1)
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
                 tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode,
-                persist=args.persist, overlap=args.overlap, kform=args.kform)
+                persist=args.persist, overlap=args.overlap, kform=args.kform,
+                trace=not args.no_trace)
     stream = t.stream
 
     def solve():
@@ -301,6 +423,8 @@ def run_gpu(args):
     for _ in range(args.warmup):
         solve()
     barrier()
+    if not args.no_trace:
+        t.trace(reset=True)  # in-graph kernel timing: the timed region only
     clk = ClockSampler(local)
     clk.start()
     l0 = t.launch_count()
@@ -338,6 +462,8 @@ def run_gpu(args):
     else:
         model_bytes = len(stats) * 5 * 8 * cells + iters * cg_iter_bytes(cells)
 
+    tr = [] if args.no_trace else t.trace(reset=True)
+
     # ---- e2e through the C ABI with host buffers (pinned)
     u_host = torch.empty(((args.nz,) if args.nz > 1 else ()) + (args.n, args.n),
                          dtype=torch.float64).pin_memory()
@@ -357,33 +483,36 @@ def run_gpu(args):
            "d2h_bytes_per_step": 8 * bx}
     t.close()
 
-    # ---- roofline of the dominant kernel: profiled solve (events per launch)
-    tp = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
-                 profile=True, tile_rows=args.tile_rows, tb_steps=args.tb_steps,
-                 check_interval=2, kform=args.kform)
-    tp.set_u(u_np)
-    pst = tp.solve(method, args.eps, args.max_iters, args.inner).stats
-    kt = tp.kernel_times()
-    tp.close()
+    # ---- roofline of the dominant kernel, from the in-graph timing of the timed region:
+    # per (kernel class, algorithmic bytes per launch) slot, the launches that did their
+    # work and their summed device time; dominant = the largest share of the kernel time
     hbm, which = peaks()
-    # dominant kernel class = the largest share of the profiled solve; its achieved
-    # bandwidth = the library's algorithmic bytes for those launches / their time
-    kkey = max(kt, key=lambda k: kt[k][0])
-    kms, kn, kbytes = kt[kkey]
-    avg_ms = kms / max(kn, 1)
-    achieved = kbytes / (kms * 1e-3) / 1e9
-    tot_ms = sum(v[0] for v in kt.values())
-    roof = {"bound": "hbm", "achieved": achieved, "peak": hbm, "unit": "GB/s",
-            "frac": achieved / hbm, "traffic": load_ncu_traffic(kkey, args.n),
-            "kernel": kkey, "algorithmic_bytes_per_launch": kbytes / max(kn, 1),
-            "avg_launch_us": avg_ms * 1e3, "launches_profiled": kn,
-            "share_of_profiled_step": kms / tot_ms if tot_ms else None,
-            "peak_source": f"MEASURED_PEAKS.json hbm_gbs ({which})",
-            "kernel_ms": {k: round(v[0], 3) for k, v in kt.items() if v[1]},
-            "kernel_gbs": {k: round(v[2] / (v[0] * 1e-3) / 1e9, 1) for k, v in kt.items()
-                           if v[1] and v[2] > 0},
-            "profiled_solve_model_gbs": sum(v[2] for v in kt.values()) / (tot_ms * 1e-3) / 1e9
-            if tot_ms else None}
+    cls = {}
+    for kname, bpl, n, kms in tr:
+        e = cls.setdefault(kname, [0.0, 0, 0.0])
+        e[0] += kms
+        e[1] += n
+        e[2] += bpl * n
+    roof = None
+    if cls:
+        tot_ms = sum(v[0] for v in cls.values())
+        kkey = max(cls, key=lambda k: cls[k][0])
+        kms, kn, kbytes = cls[kkey]
+        traffic, traffic_src = load_ncu_traffic(kkey, args.n)
+        achieved = kbytes / (kms * 1e-3) / 1e9
+        roof = {"bound": "hbm", "achieved": achieved, "peak": hbm, "unit": "GB/s",
+                "frac": achieved / hbm, "traffic": traffic, "traffic_source": traffic_src,
+                "kernel": kkey, "algorithmic_bytes_per_launch": kbytes / max(kn, 1),
+                "avg_launch_us": kms / max(kn, 1) * 1e3, "launches_timed": kn,
+                "share_of_kernel_time": kms / tot_ms, "kernel_time_of_step": tot_ms / ms,
+                "timing": "in-graph (tea_opts.trace: %globaltimer at launch start / last CTA "
+                          "end), the K timed WHILE-graph timesteps",
+                "peak_source": f"MEASURED_PEAKS.json hbm_gbs ({which})",
+                "kernel_ms": {k: round(v[0], 3) for k, v in cls.items()},
+                "kernel_avg_us": {k: round(v[0] / max(v[1], 1) * 1e3, 1) for k, v in cls.items()},
+                "kernel_gbs": {k: round(v[2] / (v[0] * 1e-3) / 1e9, 1) for k, v in cls.items()
+                               if v[2] > 0 and v[0] > 0},
+                "model_gbs_timed_region": sum(v[2] for v in cls.values()) / (ms * 1e-3) / 1e9}
 
     line = {
         "metric": metric_name(args), "value": value, "unit": "iterations/s",
@@ -399,15 +528,14 @@ def run_gpu(args):
         "matvecs_per_s": matvecs / (ms * 1e-3),
         # library-accounted algorithmic bytes (fused passes counted as
         # what they move), per iteration from the profiled solve, over the timed region
-        "hbm_gbs_model": (sum(v[2] for v in kt.values()) / max(pst["iterations"], 1)) * iters
-        / (ms * 1e-3) / 1e9,
+        "hbm_gbs_model": roof["model_gbs_timed_region"] if roof else None,
         # the same work priced at one kernel per Chebyshev step (6 streams / step):
         # an "effective bandwidth" that exceeds the HBM peak when fusion saves bytes
         "hbm_gbs_unfused_equiv": model_bytes / (ms * 1e-3) / 1e9,
         "e2e": e2e, "gpu_launches": launches, "clocks": clocks, "roofline": roof,
     }
     if rank == 0 and world == 1 and not args.no_cpu:
-        line["cpu_baseline"] = cpu_baseline(args, deck)
+        line["cpu_baseline"] = cpu_baseline(args, deck, stats)
     if rank == 0:
         print(json.dumps(line), flush=True)
     if pg is not None:
@@ -453,7 +581,8 @@ def main():
                     help="Chebyshev steps per fused HBM pass (0 auto=4, 1 = per-step kernels)")
     ap.add_argument("--loop-mode", type=int, default=0,
                     help="0 WHILE graph, 1 chunked graphs (ncu can profile), 2 eager")
-    ap.add_argument("--ref-iters", type=int, default=31)
+    ap.add_argument("--no-trace", action="store_true",
+                    help="time without the in-graph kernel timing (no roofline block)")
     ap.add_argument("--no-cpu", action="store_true")
     args = ap.parse_args()
     if args.warmup < 3:

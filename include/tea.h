@@ -31,7 +31,7 @@
 extern "C" {
 #endif
 
-#define TEA_ABI_VERSION 4
+#define TEA_ABI_VERSION 5
 
 typedef enum {
     TEA_OK = 0,
@@ -138,6 +138,14 @@ typedef struct {
                                stored Kx, Ky, 0 = auto (on). Every kernel's K is
                                bitwise the same either way (the stored faces are
                                computed by the same expression). [0] */
+    int trace;              /* 1: in-graph kernel timing. Every hot-path kernel launch
+                               (in any loop mode, inside the CUDA graphs too) stamps
+                               %globaltimer at its start (CTA 0) and adds its duration,
+                               taken by the last CTA to finish, to a per-(kernel class,
+                               algorithmic bytes) slot on the device; launches that find
+                               the solve finished (no-ops) and the finalising u update are
+                               not counted. Read with tea_trace_read(). Costs one
+                               atomicAdd per CTA per launch. 0 = off               [0] */
 } tea_opts;
 #define TEA_PERSIST_AUTO_CG (1024.0 * 1024.0)
 #define TEA_PERSIST_AUTO_CPPCG (512.0 * 512.0)
@@ -216,6 +224,14 @@ tea_status tea_set_u(tea_ctx *ctx, const double *u_host);
  * reset != 0 clears.                                                           */
 tea_status tea_kernel_times(tea_ctx *ctx, double *ms, long long *launches, double *bytes,
                             int reset);
+
+/* In-graph kernel timing (tea_opts.trace): up to `cap` slots, one per (kernel class,
+ * algorithmic bytes per launch) pair seen since tea_init, summed over this rank's blocks:
+ * kid[i] (TEA_K_*), bytes_per_launch[i] (DESIGN.md §4 model), launches[i] (launches that
+ * did their work) and ms[i] (their summed device durations). Returns the slot count (or a
+ * negative tea_status). reset != 0 zeroes the counters after reading. Host-synchronous. */
+int tea_trace_read(tea_ctx *ctx, int cap, int *kid, double *bytes_per_launch,
+                   long long *launches, double *ms, int reset);
 
 /* Kernel launches issued by the library since tea_init (all modes; graph
  * replays count their kernel nodes).                                          */

@@ -28,7 +28,8 @@ KERNELS = ["init", "residual", "spmv", "update", "cheb_first", "cheb_step", "che
            "cg1_w", "stat", "persist"]
 SYMBOLS = ["tea_version", "tea_abi_version", "tea_get_nccl_id", "tea_workspace_bytes", "tea_init",
            "tea_solve", "tea_fetch", "tea_set_u", "tea_kernel_times", "tea_launch_count",
-           "tea_finalize", "tea_last_error", "tea_block_extent", "tea_cheb_schedule"]
+           "tea_finalize", "tea_last_error", "tea_block_extent", "tea_cheb_schedule",
+           "tea_trace_read"]
 
 
 class TeaError(RuntimeError):
@@ -43,7 +44,7 @@ class Mesh(C.Structure):
                 ("zmin", C.c_double), ("zmax", C.c_double)]
 
 
-ABI_VERSION = 4  # include/tea.h TEA_ABI_VERSION (tea_opts layout)
+ABI_VERSION = 5  # include/tea.h TEA_ABI_VERSION (tea_opts layout)
 
 
 class Dist(C.Structure):
@@ -56,7 +57,7 @@ class Opts(C.Structure):
                 ("eig_margin_hi", C.c_double), ("mean_mode", C.c_int), ("loop_mode", C.c_int),
                 ("check_interval", C.c_int), ("profile", C.c_int), ("tile_rows", C.c_int),
                 ("tb_steps", C.c_int), ("tb_rows", C.c_int), ("persist", C.c_int),
-                ("overlap", C.c_int), ("kform", C.c_int)]
+                ("overlap", C.c_int), ("kform", C.c_int), ("trace", C.c_int)]
 
 
 class Stats(C.Structure):
@@ -107,6 +108,7 @@ def lib(build_if_needed: bool = True):
     L.tea_last_error.restype = C.c_char_p
     L.tea_block_extent.argtypes = [C.POINTER(Mesh), i, i, i] + [C.POINTER(C.c_int)] * 4
     L.tea_cheb_schedule.argtypes = [i, i, vp, i]
+    L.tea_trace_read.argtypes = [vp, i, vp, vp, vp, vp, i]
     _lib = L
     return L
 
@@ -181,7 +183,8 @@ class Tea:
                  presteps: int = 30, eig_margins=(0.95, 1.05), mean_mode: int = 0,
                  loop_mode: int = 0, check_interval: int = 0, profile: bool = False,
                  tile_rows: int = 0, tb_steps: int = 0, tb_rows: int = 0, persist: int = 0,
-                 overlap: int = 0, kform: int = 0, device=None, stream=None):
+                 overlap: int = 0, kform: int = 0, trace: bool = False, device=None,
+                 stream=None):
         import torch
         if not torch.cuda.is_available():
             raise RuntimeError("paper_conf_cluster_mcintosh_smithm17_b200 needs a CUDA device "
@@ -202,7 +205,7 @@ class Tea:
                               C.cast(self._nccl_id, C.c_void_p) if self._nccl_id else None)
         self.opts = Opts(presteps, eig_margins[0], eig_margins[1], mean_mode, loop_mode,
                          check_interval, 1 if profile else 0, tile_rows, tb_steps, tb_rows,
-                         persist, overlap, kform)
+                         persist, overlap, kform, 1 if trace else 0)
         with torch.cuda.device(self.device):
             nbytes = workspace_bytes(mesh, self._dist)
             self.workspace = torch.empty(nbytes, dtype=torch.uint8, device=self.device)
@@ -252,6 +255,20 @@ class Tea:
         by = (C.c_double * len(KERNELS))()
         self.L.tea_kernel_times(self.ctx, ms, n, by, 1 if reset else 0)
         return {k: (ms[i], n[i], by[i]) for i, k in enumerate(KERNELS)}
+
+    def trace(self, reset=False):
+        """In-graph kernel timing (trace=True): [(kernel class, algorithmic bytes per launch,
+        launches, total ms)] -- device durations of the launches that did their work, taken
+        inside whatever graphs / loop mode the solve ran in."""
+        cap = 64
+        kid = (C.c_int * cap)()
+        by = (C.c_double * cap)()
+        n = (C.c_longlong * cap)()
+        ms = (C.c_double * cap)()
+        k = self.L.tea_trace_read(self.ctx, cap, kid, by, n, ms, 1 if reset else 0)
+        if k < 0:
+            raise TeaError(k, self.L.tea_last_error(self.ctx).decode())
+        return [(KERNELS[kid[i]], by[i], n[i], ms[i]) for i in range(min(k, cap))]
 
     def launch_count(self) -> int:
         return int(self.L.tea_launch_count(self.ctx))

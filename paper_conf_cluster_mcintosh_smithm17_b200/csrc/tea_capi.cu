@@ -79,6 +79,9 @@ BlockLayout layout_block(const tea_mesh &m, int px, int py, int d, int b) {
     size_t off = L.field_bytes * F_COUNT;
     L.scalars_off = off;
     off += round_up(sizeof(Scalars), 256);
+    // two values per CTA of the largest grid any reducing launch can use: 2D stencil and
+    // pointwise tiles down to one row (tile_rows = 1) on the extended region; 3D stencil
+    // tiles down to one plane, 3D pointwise tiles one row x one plane
     L.partials_cap = 2 * (size_t)std::max(max_ctas(L.bx + 2 * d + 2, L.by + 2 * d + 2),
                                           L.nz > 1 ? max_ctas3(L.bx, L.by, L.nz) : 0);
     L.partials_cap = std::max(L.partials_cap, (size_t)6 * 1024);  // k_persist: 2 x 3 x CTAs
@@ -148,6 +151,9 @@ struct tea_ctx {
     std::map<long long, int> graph_kernels;
     // capture state
     cudaGraphConditionalHandle cond = 0;
+    // in-graph kernel timing (tea_opts.trace): slot i times launches of (kid, bytes)
+    std::vector<std::pair<int, double>> tslots;
+    int cur_tslot = -1;
     int ty_override = 0;
     int coef_slot = -1;  // constant-memory coefficient slot of the fused passes
 };
@@ -200,13 +206,39 @@ KArgs kargs(tea_ctx *c, const BlockCtx &b, bool set_cond = false) {
     a.g = (b.L.nz == 1 && c->opts.kform >= 0) ? b.f[F_KZ] : nullptr;
     a.hrx = 0.5 * c->rx;
     a.hry = 0.5 * c->ry;
+    a.tslot = c->cur_tslot;
     return a;
+}
+
+// kernel classes whose kernels carry the trace_begin / trace_end hooks
+bool traced_kid(int kid) {
+    switch (kid) {
+        case TEA_K_RESIDUAL: case TEA_K_SPMV: case TEA_K_UPDATE: case TEA_K_CHEB_FIRST:
+        case TEA_K_CHEB_STEP: case TEA_K_CHEB_LAST: case TEA_K_TB_FIRST: case TEA_K_TB_MID:
+        case TEA_K_TB_LAST: case TEA_K_BJ: case TEA_K_CG1: case TEA_K_CG1W: case TEA_K_STAT:
+            return true;
+        default:
+            return false;
+    }
+}
+int trace_slot(tea_ctx *c, int kid, double bytes) {
+    if (!c->opts.trace || !traced_kid(kid)) return -1;
+    for (size_t i = 0; i < c->tslots.size(); ++i)
+        if (c->tslots[i].first == kid && c->tslots[i].second == bytes) return (int)i;
+    if ((int)c->tslots.size() >= kTraceSlots) return -1;  // full: this pair goes untimed
+    c->tslots.emplace_back(kid, bytes);
+    return (int)c->tslots.size() - 1;
 }
 
 // Issue one kernel launch (profiled with an event pair when profiling). `bytes` =
 // the launch's algorithmic HBM bytes, accumulated per kernel class.
 template <class F>
 void K(tea_ctx *c, int kid, double bytes, F &&f) {
+    c->cur_tslot = trace_slot(c, kid, bytes);
+    struct Reset {
+        int &v;
+        ~Reset() { v = -1; }
+    } reset_{c->cur_tslot};
     if (c->profiling) {
         if (c->evnext + 2 > c->evpool.size()) {
             for (int i = 0; i < 256; ++i) {
@@ -246,9 +278,17 @@ Launch plan(tea_ctx *c, const Region &R) {
     return plan_stencil(R, c->opts.tile_rows > 0 ? c->opts.tile_rows : c->ty_override, 1184);
 }
 // stencil kernels: 2D march over rows, or the 3D march over planes
+// every reducing launch writes NV <= 2 partials per CTA into the block's scratch
+const Launch &checked(const BlockCtx &b, const Launch &L) {
+    const size_t ctas = (size_t)L.grid.x * L.grid.y * L.grid.z;
+    if (2 * ctas > b.L.partials_cap)
+        fail(TEA_ERR_STATE, "launch of %zu CTAs exceeds the reduction scratch (%zu partials)",
+             ctas, b.L.partials_cap);
+    return L;
+}
 Launch plan_st(tea_ctx *c, const BlockCtx &b, const Region &R) {
-    if (b.L.nz > 1) return plan_stencil3(R, b.L.nz, c->opts.tile_rows);
-    return plan(c, R);
+    if (b.L.nz > 1) return checked(b, plan_stencil3(R, b.L.nz, c->opts.tile_rows));
+    return checked(b, plan(c, R));
 }
 // the SpMV: large 2D blocks (where the default tile is the 32-row cap) get wave-fitted tiles
 Launch plan_spmv(tea_ctx *c, const BlockCtx &b, const Region &R) {
@@ -259,12 +299,12 @@ Launch plan_spmv(tea_ctx *c, const BlockCtx &b, const Region &R) {
         // 4776 -> 4965 GB/s, profiles/r01k_tz3.txt)
         const int cols = (int)(L.grid.x * L.grid.y);
         const int gz = std::max(1, 592 / std::max(cols, 1));
-        return plan_stencil3(R, b.L.nz, std::max(4, (b.L.nz + gz - 1) / gz));
+        return checked(b, plan_stencil3(R, b.L.nz, std::max(4, (b.L.nz + gz - 1) / gz)));
     }
     if (b.L.nz > 1 || c->opts.tile_rows > 0 || c->ty_override > 0 || L.ty < 32) return L;
     const int ty = spmv_wave_rows(R.j1 - L.jstart, R.k1 - R.k0);
     // one reduction partial per CTA must fit the block's scratch (fewer CTAs: always true)
-    return plan_stencil(R, ty, 0);
+    return checked(b, plan_stencil(R, ty, 0));
 }
 // pointwise kernels: the 2D tiling of one plane, planes on grid.z
 Launch plan_pw(tea_ctx *c, const BlockCtx &b, const Region &R) {
@@ -274,7 +314,7 @@ Launch plan_pw(tea_ctx *c, const BlockCtx &b, const Region &R) {
     const int tr = c->opts.tile_rows > 0 ? c->opts.tile_rows : c->ty_override;
     Launch L = b.L.nz > 1 ? plan_stencil(R, tr > 0 ? tr : 8, 1184) : plan(c, R);
     L.grid.z = b.L.nz;
-    return L;
+    return checked(b, L);
 }
 
 // ------------------------------------------------------------------ reductions
@@ -289,6 +329,8 @@ void reduce(tea_ctx *c, int first, int n) {
     }
     if (c->nranks > 1) {
         double *p = &c->blocks[0].S->red_pw + first;
+        K(c, TEA_K_SCALAR, 0.0,
+          [&] { launch_mask_done(c->blocks[0].S, first, n, c->rank != 0, c->stream); });
         NK(ncclAllReduce(p, p, n, ncclDouble, ncclSum, c->comm, c->stream));
     }
 }
@@ -1023,6 +1065,14 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
     }
     reduce(c, 1, 2);
     if (method == TEA_BJCG) {  // z = M^{-1} r, r.z, r.r (no update)
+        // Thomas coefficients of the strips (they depend on A only) into the two fields
+        // block Jacobi never uses (F_BJC = Z2, F_BJD = Z3): ~0.1 ms at 4096^2, no HBM kept
+        // for them across solves of other methods
+        for (auto &b : c->blocks)
+            K(c, TEA_K_INIT, 0.0, [&] {
+                launch_bj_setup(kargs(c, b), b.owned(), b.f[F_KX], b.f[F_KY], b.f[F_BJC],
+                                b.f[F_BJD], c->stream);
+            });
         for (auto &b : c->blocks)
             K(c, TEA_K_BJ, sbytes(b, 5), [&] {
                 launch_bj(kargs(c, b), b.owned(), false, false, b.f[F_W], b.f[F_R0], b.f[F_Z0],
@@ -1269,13 +1319,36 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
         if (o.persist < -1 || o.persist > 1) fail(TEA_ERR_ARG, "bad persist");
         if (o.overlap < -1 || o.overlap > 1) fail(TEA_ERR_ARG, "bad overlap");
         if (o.kform < -1 || o.kform > 1) fail(TEA_ERR_ARG, "bad kform");
+        if (o.trace < 0 || o.trace > 1) fail(TEA_ERR_ARG, "bad trace");
         // NCCL kernels inside a WHILE-conditional graph body are not a supported
         // capture target: multi-process runs use chunked graphs (same kernels).
         if (nranks > 1 && o.loop_mode == 0) o.loop_mode = 1;
         c->opts = o;
-        const long long ncell = (long long)mesh->nx * mesh->ny * (mesh->nz > 1 ? mesh->nz : 1);
-        for (long long i = 0; i < ncell; i += 1 + ncell / 4096)
-            if (!(density[i] > 0.0)) fail(TEA_ERR_ARG, "density must be > 0");
+        // every cell this rank stages (its blocks plus the margin; all of a 3D mesh): a
+        // density <= 0 would silently become an insulating internal boundary
+        {
+            const int bpr0 = px * py / nranks, m0 = d + 1;
+            const long long nzc = mesh->nz > 1 ? mesh->nz : 1;
+            for (int bi = rank * bpr0; bi < (rank + 1) * bpr0; ++bi) {
+                const BlockLayout L0 = layout_block(*mesh, px, py, d, bi);
+                const int x0 = nzc > 1 ? 0 : std::max(0, L0.gx0 - m0);
+                const int x1 = nzc > 1 ? mesh->nx : std::min(mesh->nx, L0.gx1 + m0);
+                const int y0 = nzc > 1 ? 0 : std::max(0, L0.gy0 - m0);
+                const int y1 = nzc > 1 ? mesh->ny : std::min(mesh->ny, L0.gy1 + m0);
+                for (long long l = 0; l < nzc; ++l)
+                    for (int k = y0; k < y1; ++k) {
+                        const size_t row = ((size_t)l * mesh->ny + k) * mesh->nx;
+                        for (int j = x0; j < x1; ++j) {
+                            const double rh = density[row + j], en = energy[row + j];
+                            if (!(rh > 0.0) || !std::isfinite(rh))
+                                fail(TEA_ERR_ARG, "density must be finite and > 0 (cell %d,%d,%lld)",
+                                     j, k, l);
+                            if (!std::isfinite(en))
+                                fail(TEA_ERR_ARG, "energy must be finite (cell %d,%d,%lld)", j, k, l);
+                        }
+                    }
+            }
+        }
 
         c->user_stream = (cudaStream_t)cuda_stream;
         CK(cudaStreamCreateWithFlags(&c->stream, cudaStreamNonBlocking));
@@ -1371,10 +1444,6 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
                                    b.f[F_KX], b.f[F_KY], b.f[F_KZ], owned, all, kxr, kyr, gall,
                                    0.5 * c->rx, 0.5 * c->ry, o.mean_mode, c->stream);
             });
-            K(c.get(), TEA_K_INIT, 0.0, [&] {
-                launch_bj_setup(kargs(c.get(), b), owned, b.f[F_KX], b.f[F_KY], b.f[F_BJC],
-                                b.f[F_BJD], c->stream);
-            });
             // the staging fields are solver fields with zero halos: clear them again
             CK(cudaMemsetAsync(ws + F_W * L.field_bytes, 0, L.field_bytes, c->stream));
             CK(cudaMemsetAsync(ws + F_Z0 * L.field_bytes, 0, L.field_bytes, c->stream));
@@ -1461,6 +1530,42 @@ tea_status tea_kernel_times(tea_ctx *ctx, double *ms, long long *launches, doubl
         std::memset(ctx->kbytes, 0, sizeof ctx->kbytes);
     }
     return TEA_OK;
+}
+
+int tea_trace_read(tea_ctx *ctx, int cap, int *kid, double *bytes_per_launch,
+                   long long *launches, double *ms, int reset) {
+    if (!ctx || cap < 0) return TEA_ERR_ARG;
+    try {
+        if (ctx->failed) fail(TEA_ERR_STATE, "context failed: %s", ctx->err.c_str());
+        const int n = (int)ctx->tslots.size();
+        std::vector<unsigned long long> ns(n, 0ull), cnt(n, 0ull);
+        std::vector<unsigned long long> h(2 * kTraceSlots);
+        CK(cudaStreamSynchronize(ctx->stream));
+        for (auto &b : ctx->blocks) {
+            CK(cudaMemcpy(h.data(), b.S->trace_ns, sizeof(unsigned long long) * kTraceSlots,
+                          cudaMemcpyDeviceToHost));
+            CK(cudaMemcpy(h.data() + kTraceSlots, b.S->trace_n,
+                          sizeof(unsigned long long) * kTraceSlots, cudaMemcpyDeviceToHost));
+            for (int i = 0; i < n; ++i) {
+                ns[i] += h[i];
+                cnt[i] += h[kTraceSlots + i];
+            }
+            if (reset) {
+                CK(cudaMemset(b.S->trace_ns, 0, sizeof(unsigned long long) * kTraceSlots));
+                CK(cudaMemset(b.S->trace_n, 0, sizeof(unsigned long long) * kTraceSlots));
+            }
+        }
+        for (int i = 0; i < n && i < cap; ++i) {
+            if (kid) kid[i] = ctx->tslots[i].first;
+            if (bytes_per_launch) bytes_per_launch[i] = ctx->tslots[i].second;
+            if (launches) launches[i] = (long long)cnt[i];
+            if (ms) ms[i] = 1e-6 * (double)ns[i];
+        }
+        return n;
+    } catch (const TeaError &e) {
+        ctx->err = e.msg;
+        return e.st;
+    }
 }
 
 long long tea_launch_count(const tea_ctx *ctx) { return ctx ? ctx->launches : 0; }

@@ -320,6 +320,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             return;
         }
     }
+    trace_begin(a);
     const double2 z0 = make_double2(0.0, 0.0);
     // One warp allocates the CTA's TMEM columns; warp w then owns lanes 32(w%4).. and a
     // 128-column group per 4 warps: per thread a private ring of D row slots (tm_st16).
@@ -594,6 +595,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     } else if (FUSE) {
         if (blockIdx.x == 0 && blockIdx.y == 0 && blockIdx.z == 0 && threadIdx.x == 0) S->alpha_prev = alpha;
     }
+    trace_end(a);
 }
 
 int tb_out_cols(int M) {
@@ -612,11 +614,13 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
     const int nstrips = (width + G::OW - 1) / G::OW;
     dim3 grid((nstrips + kTbW - 1) / kTbW, (R.k1 - R.k0 + ty - 1) / ty);
     constexpr size_t smem = tb_smem_bytes();
-    static bool attr = false;  // per instantiation
-    if (!attr) {
+    // > 48 KB of dynamic shared memory needs the attribute, set once per device
+    static std::atomic<unsigned long long> attr{0ull};  // per instantiation: device bit mask
+    const unsigned long long bit = 1ull << tea_device();
+    if (!(attr.load() & bit)) {
         cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST, KG>,
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        attr = true;
+        attr.fetch_or(bit);
     }
     k_cheb_tb<M, FIRST, FUSE, LAST, KG><<<grid, kTbT, smem, st>>>(
         rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, a, R, Dd, ty, jlim, step0, restart ? 1 : 0);
@@ -655,11 +659,12 @@ int tb_max_steps() { return 5; }
 // CTAs are alike, so a launch costs ~ waves x (ty + 2M) with waves = ceil(ctas / slots).
 // Pick ty minimising that (slots = SMs x resident CTAs per SM of this kernel).
 int tb_auto_rows(int M, int width, int height) {
-    static int slots[8] = {};
+    static std::atomic<int> slot_cache[kMaxDev][8];
     M = M < 1 ? 1 : (M > kTbMaxSteps ? kTbMaxSteps : M);
-    if (!slots[M]) {
-        int dev = 0, nsm = 148, per = 0;
-        cudaGetDevice(&dev);
+    const int dev = tea_device();
+    int slots_m = slot_cache[dev][M].load();
+    if (!slots_m) {
+        int nsm = 148, per = 0;
         cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, dev);
         const size_t smem = tb_smem_bytes();
         cudaError_t e = cudaSuccess;
@@ -676,8 +681,11 @@ int tb_auto_rows(int M, int width, int height) {
 #undef OCC
         }
         if (e != cudaSuccess || per < 1) per = 1;
-        slots[M] = nsm * per;
+        slots_m = nsm * per;
+        slot_cache[dev][M].store(slots_m);
     }
+    int slots[8] = {};
+    slots[M] = slots_m;
     const int ow = tb_out_cols(M);
     const int gx = ((width + ow - 1) / ow + kTbW - 1) / kTbW;
     int best = height, bestc = 0x7fffffff;

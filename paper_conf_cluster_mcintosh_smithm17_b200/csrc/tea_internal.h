@@ -5,8 +5,19 @@
 #include <cuda_runtime.h>
 #include <cstddef>
 #include <cstdint>
+#include <atomic>
 
 namespace tea {
+
+// Per-device host caches (occupancy-derived tile plans, function attributes): a process may
+// drive contexts on several GPUs, so every cache is indexed by the current device and
+// filled idempotently (atomics: concurrent first uses compute the same value).
+constexpr int kMaxDev = 64;
+inline int tea_device() {
+    int d = 0;
+    cudaGetDevice(&d);
+    return d < 0 ? 0 : (d >= kMaxDev ? kMaxDev - 1 : d);
+}
 
 constexpr int kMaxPre = 512;   // presteps cap (Lanczos history length)
 constexpr int kMaxS = 64;      // Chebyshev inner steps cap
@@ -14,6 +25,7 @@ constexpr int kWarps = 4;      // warps per CTA in the stencil / pointwise kerne
 constexpr int kThreads = 32 * kWarps;
 constexpr int kStrip = 64;     // columns per warp (32 lanes x double2)
 constexpr int kCtaCols = kWarps * kStrip;
+constexpr int kTraceSlots = 32;  // (kernel class, bytes per launch) pairs timed in-graph
 
 // Device-side solver state, one copy per local block (all copies evolve
 // identically: every decision is taken from globally reduced scalars).
@@ -46,6 +58,11 @@ struct Scalars {
     double cheb_a[kMaxS], cheb_b[kMaxS];                 // Saad 12.1 a_i, b_i
     double cheb_cx[kMaxS], cheb_cz[kMaxS], cheb_cr[kMaxS], cheb_ca[kMaxS];  // folded, §4.3
     double alpha_hist[kMaxPre], beta_hist[kMaxPre];
+    // in-graph kernel timing (tea_opts.trace): per trace slot, the %globaltimer of the
+    // current launch's start (CTA 0), the summed launch durations (ns), the launch count, and
+    // the completion ticket. Launches that find the solve finished (no-ops) are not counted.
+    unsigned long long trace_t0[kTraceSlots], trace_ns[kTraceSlots], trace_n[kTraceSlots];
+    unsigned trace_ticket[kTraceSlots];
 };
 
 enum { DS_RUNNING = 0, DS_CONVERGED = 1, DS_LIMIT = 2, DS_BREAKDOWN = 3, DS_EIGFAIL = 4 };
@@ -58,8 +75,10 @@ struct Region {
 // Field indices inside a block's workspace.
 enum Field {
     F_U0 = 0, F_U, F_KX, F_KY, F_KZ, F_R0, F_R1, F_P0, F_P1, F_W, F_Z0, F_Z1, F_Z2, F_Z3,
-    F_BJC, F_BJD,  // block-Jacobi Thomas coefficients c'_i and 1/den_i
-    F_COUNT
+    F_COUNT,
+    // block-Jacobi Thomas coefficients c'_i and 1/den_i: recomputed at the start of every
+    // block-Jacobi solve into two fields that method never uses
+    F_BJC = F_Z2, F_BJD = F_Z3
 };
 
 // Launch geometry of one stencil / pointwise launch.
@@ -89,7 +108,39 @@ struct KArgs {
     // Ky(j,k) = hry (g(j,k-1) + g(j,k)). g == nullptr: the kernels read the stored Kx, Ky.
     const double *g;
     double hrx, hry;
+    int tslot;  // in-graph timing slot of this launch (tea_opts.trace), -1 = not traced
 };
+
+// In-graph kernel timing (tea_opts.trace): CTA 0 stamps the start, the last
+// CTA to finish adds the launch's duration to its slot. trace_end must be reached by every
+// thread of every CTA of a traced launch.
+__device__ __forceinline__ unsigned long long tea_gtimer() {
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    return t;
+}
+__device__ __forceinline__ void trace_begin(const KArgs &a) {
+    if (a.tslot >= 0 && blockIdx.x == 0 && blockIdx.y == 0 && blockIdx.z == 0 &&
+        threadIdx.x == 0) {
+        a.S->trace_t0[a.tslot] = tea_gtimer();
+        __threadfence();
+    }
+}
+__device__ __forceinline__ void trace_end(const KArgs &a) {
+    if (a.tslot < 0) return;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        const unsigned n = gridDim.x * gridDim.y * gridDim.z;
+        if (atomicAdd(&a.S->trace_ticket[a.tslot], 1u) == n - 1u) {
+            const unsigned long long t1 = tea_gtimer();
+            volatile unsigned long long *t0 = a.S->trace_t0;
+            a.S->trace_ns[a.tslot] += t1 - t0[a.tslot];
+            a.S->trace_n[a.tslot] += 1ull;
+            a.S->trace_ticket[a.tslot] = 0u;
+        }
+    }
+}
 
 Launch plan_stencil(const Region &R, int ty_req, int ncta_target);
 // 3D stencil geometry: CTA = 4 warps on 4 consecutive rows of one 64-column strip,
@@ -131,6 +182,7 @@ void launch_scalars(const KArgs &a, int mode, double eps, int it_limit, int max_
                     double mlo, double mhi, cudaStream_t st);
 void launch_combine(Scalars *const *S_dev_list, int nblocks, int nvals, int first_slot,
                     cudaStream_t st);
+void launch_mask_done(Scalars *S, int first, int nvals, bool zero, cudaStream_t st);
 void launch_pack(const double *const *fields, int nf, int pitch, const int *boxes,
                  int nbox, double *buf, cudaStream_t st);
 void launch_unpack(double *const *fields, int nf, int pitch, const int *boxes, int nbox,

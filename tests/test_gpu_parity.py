@@ -37,12 +37,21 @@ def rel_err(a, b):
 
 
 def field_err(a, b, kind):
-    """Pipe decks: pointwise relative error. Random decks (u = rho e spans six decades
-    cell to cell, so a cell's value can be a 1e-6 remnant of cancelling O(1) terms):
-    max abs error over max |u| (parity metric)."""
-    if kind == "pipe":
-        return rel_err(a, b)
-    return float(np.max(np.abs(a - b)) / np.max(np.abs(b)))
+    """The north_star metric on every deck: max pointwise relative error (u > 0 on the pipe
+    and on the random decks; measured on the random decks: <= 3e-12 where the pipe gives
+    ~1e-13, profiles/r02_random_metric.txt). `kind` is kept for the call sites."""
+    return rel_err(a, b)
+
+
+def residual_bound(ora, deck, *fields):
+    """Sum of the TRUE residual norms ||u^n - A u||_2 of the given fields (oracle operator).
+    lambda_min(A) >= 1 (A = I + dt L, L positive semidefinite: pinned in
+    tests/test_oracle_operator.py), so ||u - u*||_2 <= ||u^n - A u||_2 for ANY field u, and
+    two fields differ by at most the sum at every cell (reading R22)."""
+    rx, ry = ora.mesh_r(deck)
+    Kx, Ky = ora.face_coefficients(deck.nx, deck.ny, rx, ry, deck.density)
+    u0 = deck.density * deck.energy
+    return sum(float(np.linalg.norm(u0 - ora.apply_A(Kx, Ky, u))) for u in fields)
 
 
 def gpu_run(tea, deck, steps=1, **kw):
@@ -252,6 +261,9 @@ def test_multiblock_fixed_iterations(tea, ora, px, py, d):
                             method=method, eps=0.0, max_iters=k, inner_steps=6)
         assert st_g[0]["iterations"] == k
         assert field_err(u_g, u_o, "random") <= 1e-12
+        # the reported residual norm is the global one (reductions are not replayed after
+        # the solve ends)
+        assert st_g[0]["rnorm"] == pytest.approx(st_o[0]["rnorm"], rel=1e-9)
 
 
 # ---------------------------------------------------------------- fused passes
@@ -276,21 +288,26 @@ def test_fused_passes_converged(tea, ora, tb, s):
 def test_fused_passes_fixed_iterations(tea, ora, kind, nx, ny, tb):
     """30 presteps + 3 outer iterations, eps = 0, on ragged shapes: the fused passes
     agree with the one-kernel-per-step path to rounding (1e-12), and with the oracle
-    to 1e-12 where the mid-solve iterate is well conditioned (pipe, 2D random decks).
-    On the 1-cell-wide meshes the first PCG iterates are sensitive to the
-    preconditioner's rounding (the Chebyshev polynomial grows outside the estimated
-    interval): both GPU paths differ from the oracle's Saad-form preconditioner by up to
-    5e-7 after one outer iteration, shrinking to 3e-15 at convergence
-    (tools/diag_1col.py) -- there the converged tests apply."""
+    to 1e-12 on 2D meshes. On the 1-cell-wide random meshes A has an eigenvalue 1.0006
+    next to its exact lambda_min = 1 (a nearly insulated stretch of the random density),
+    below the estimated Chebyshev interval [1.08, 58]: the mid-solve iterates carry
+    rounding-driven components in that near-null pair that the oracle's Saad-form and the
+    GPU's three-term preconditioner round differently (measured 3e-8 / 7e-8 pointwise after
+    one outer iteration, 3e-15 at convergence: profiles/r02_random_metric.txt). There the
+    oracle comparison is the rigorous computed bound of reading R22 -- every cell within
+    the sum of the two true residual norms -- and the converged tests give the 1e-10 bar."""
     deck = deck_of(kind, nx, ny, seed=4, dt=0.04)
     kw = dict(method=1, eps=0.0, max_iters=33, inner_steps=7)
     u_1, st_1 = gpu_run(tea, deck, tb_steps=1, **kw)
     u_g, st_g = gpu_run(tea, deck, tb_steps=tb, **kw)
     assert st_g[0]["iterations"] == st_1[0]["iterations"] == 33
     assert field_err(u_g, u_1, "random") <= 1e-12
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
     if min(nx, ny) > 1:
-        u_o, st_o, _ = ora.run(deck, steps=1, **kw)
         assert field_err(u_g, u_o, kind) <= 1e-12
+    else:
+        assert float(np.max(np.abs(u_g - u_o))) <= residual_bound(ora, deck, u_g, u_o)
+        assert st_g[0]["rnorm"] == pytest.approx(st_o[0]["rnorm"], rel=1e-3)
     kw = dict(method=1, eps=1e-13, max_iters=5000, inner_steps=7)
     u_o, st_o, _ = ora.run(deck, steps=1, **kw)
     u_c, st_c = gpu_run(tea, deck, tb_steps=tb, **kw)

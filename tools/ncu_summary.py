@@ -12,6 +12,7 @@ import sys
 from collections import defaultdict
 
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
 
 
 def raw_rows(rep):
@@ -92,6 +93,14 @@ def main():
     agg = launch_list(ll) if os.path.exists(ll) else {}
     if os.path.exists(ll):
         subprocess.call(["cp", ll, os.path.join(prof, f"{tag}_launches_bench{n}.csv")])
+    # the same launch list with --cache-control none (L2 not flushed between kernels: each
+    # kernel pays the write-back of its predecessor's dirty lines, as inside the bench)
+    llw = os.path.join(src, "launches_warm.csv")
+    aggw = launch_list(llw) if os.path.exists(llw) else {}
+    if os.path.exists(llw):
+        subprocess.call(["cp", llw, os.path.join(prof, f"{tag}_launches_warm_bench{n}.csv")])
+    import bench
+    shash = bench.source_hash()
     # traffic per launch for bench.py: average over the captured launches of each class
     key = {"k_cheb_tb<5, 1, 1, 0>": "tb_first", "k_cheb_tb<5, 0, 0, 1>": "tb_last",
            "k_cheb_tb<5, 1, 1, 0, 1>": "tb_first", "k_cheb_tb<5, 0, 0, 1, 1>": "tb_last",
@@ -110,11 +119,19 @@ def main():
         ent["algorithmic_bytes_per_launch"] = {"spmv": 7, "tb_first": 6, "tb_last": 5}[cls] * 8 * n * n
         ent["kernel"] = v[0][1]
         ent["round"] = tag[1:] if tag.startswith("r") else tag
+        ent["source_hash"] = shash
+        ent["capture"] = f"ncu --set full, gpurun_out/prof_{tag}, summary profiles/{tag}_ncu_summary.md"
     json.dump(traffic, open(tp, "w"), indent=1)
     tot = sum(a[1] for a in agg.values()) or 1.0
-    lines = ["| kernel | launches | mean us | share |", "|---|---|---|---|"]
+    totw = sum(a[1] for a in aggw.values()) or 1.0
+    lines = [f"source hash {shash}", "",
+             "| kernel | launches | mean us (cold L2) | share | mean us (warm L2) | share |",
+             "|---|---|---|---|---|---|"]
     for k, (c, s) in sorted(agg.items(), key=lambda x: -x[1][1]):
-        lines.append(f"| {k} | {c} | {s / c / 1e3 if s > 1e4 else s / c:.1f} | {s / tot:.3f} |")
+        cw, sw = aggw.get(k, (0, 0.0))
+        mw = ((sw / cw / 1e3 if s > 1e4 else sw / cw) if cw else float("nan"))
+        lines.append(f"| {k} | {c} | {s / c / 1e3 if s > 1e4 else s / c:.1f} | {s / tot:.3f} | "
+                     f"{mw:.1f} | {sw / totw:.3f} |")
     lines += ["", "| kernel | us | DRAM MB (r+w) | L1TEX lsu wavefronts % | issue % | fp64 pipe % |"
               " warps active % | regs | top stalls (per issue) |", "|---|---|---|---|---|---|---|---|---|"]
     for k in full:

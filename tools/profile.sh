@@ -11,6 +11,11 @@ python -c "import __graft_entry__ as g; g.build()" > $OUT/build.log 2>&1
 timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none -c 3000 --csv \
    --log-file $OUT/launches.csv python bench.py --n $N --steps 1 --warmup 3 --no-cpu \
    --loop-mode 2 > $OUT/bench_under_ncu.log 2>&1
+# 1b) the same list with the L2 left as the previous kernel left it (--cache-control none):
+#    what the bench's in-graph timing sees (write-back of the predecessor's dirty lines)
+timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none --cache-control none \
+   -c 3000 --csv --log-file $OUT/launches_warm.csv python bench.py --n $N --steps 1 --warmup 3 \
+   --no-cpu --loop-mode 2 > $OUT/bench_under_ncu_warm.log 2>&1
 # 2) full sets: the fused Chebyshev passes of the first outer iterations (skip the two
 #    restart passes) and two SpMVs of the PCG phase
 timeout 900 ncu --set full --clock-control none --import-source on \
