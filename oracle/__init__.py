@@ -26,7 +26,7 @@ _SRC = os.path.join(_HERE, "tea_oracle.c")
 _LIB = os.path.join(_HERE, "libtea_oracle.so")
 CFLAGS = ["-O2", "-ffp-contract=off", "-fno-fast-math", "-std=c99", "-fPIC", "-shared"]
 
-CG, CPPCG, BJCG, CG1, JACOBI, CHEBY, CPPCG1 = 0, 1, 2, 3, 4, 5, 6
+CG, CPPCG, BJCG, CG1, JACOBI, CHEBY, CPPCG1, CPPCG1F = 0, 1, 2, 3, 4, 5, 6, 7
 OK, NOT_CONVERGED, ERR_ARG, ERR_BREAKDOWN = 0, 1, -1, -4
 PRESTEPS = 30  # reading R6
 

@@ -37,7 +37,8 @@ namespace tea {
 constexpr int kTbW = TEA_TB_WARPS;
 constexpr int kTbT = 32 * kTbW;
 #ifndef TEA_TB_CPA
-#define TEA_TB_CPA 4  // rows of cp.async input staging ahead of the march (first pass)
+#define TEA_TB_CPA 6  // rows of cp.async input staging ahead of the march (first pass): 4 -> 6
+                      // rows, 184 -> 164 us at 4096^2 (profiles/r02_knobs_ab.txt)
 #endif
 constexpr int kTbNS = 5;  // staged streams per row (X, W or z_{i-2}, r, Kx, Ky)
 
@@ -268,10 +269,36 @@ constexpr size_t tb_smem_bytes() {
                : 48u * 1024u;
 }
 
+#ifndef TEA_TB_SHARE
+#define TEA_TB_SHARE 0
+#endif
+// TEA_TB_SHARE (measured, not kept -- DESIGN.md §4.4): the warps of a CTA march adjacent
+// 64-column strips and hand each other their strip-edge values through shared memory once per
+// row (one CTA barrier per row), so a CTA loses MR columns per side instead of every warp
+// (244 of 256 columns at M = 5 instead of 4 x 54). Bitwise the same results, but the barrier
+// couples the 4 warps' latency chains: 274 vs 179 us per pass at 4096^2
+// (profiles/r02_tb_share_ab.txt).
+constexpr bool kTbShare = TEA_TB_SHARE != 0;
+// Strip geometry (unshared): a warp's 64 columns output [SH, SH + OW); strips start SH
+// before the region at a stride of OW. 1 (default): SH = MR = M rounded up to even,
+// OW = 64 - 2 MR (52 at M = 5). 0: OW = 64 - 2M (54 at M = 5: fewer redundant columns but
+// 215 vs 184 us per first pass at 4096^2 -- strip starts at 8 offsets mod 128 B instead of 4,
+// profiles/r02_knobs_ab.txt). 2: SH = 8, OW = 48 (M <= 8): every strip starts on a 32-B
+// sector, x1.33 redundant work.
+#ifndef TEA_TB_GEOM
+#define TEA_TB_GEOM 1
+#endif
 template <int M>
 struct TbGeom {
-    static constexpr int MR = (M + 1) & ~1;  // margin, even (double2 alignment)
-    static constexpr int OW = kStrip - 2 * MR;  // output columns per warp strip
+    static constexpr int MR = (M + 1) & ~1;  // first strip's shift: >= M, even (double2 loads)
+    // output columns per warp strip (unshared): [M, 64 - M) -- the stride 64 - 2M is even, so
+    // every strip still starts on a double2 (M = 5: 54 columns, x1.185 redundant work)
+    static constexpr int SH = TEA_TB_GEOM == 2 ? 8 : MR;
+    static constexpr int OW = TEA_TB_GEOM == 0 ? kStrip - 2 * M
+                              : (TEA_TB_GEOM == 2 ? 48 : kStrip - 2 * MR);
+    static_assert(SH >= M && SH + OW <= kStrip - M && OW % 2 == 0, "strip geometry");
+    // output columns per CTA
+    static constexpr int OWC = kTbShare ? kTbW * kStrip - 2 * MR : kTbW * OW;
     static constexpr int D = 8;  // TMEM ring depth (rows k-M-1..k fit for M <= 6); a power of
                                  // two so slots are (head - t) & 7
 };
@@ -342,18 +369,24 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     for (int d = 0; d < D; ++d) tm_st16(tm + 16u * d, z0, z0, z0, z0);  // zero ring
 
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    const int strip = blockIdx.x * kTbW + warp;
     // strips tile the output region R (which may reach into the halo on sides with a
-    // neighbour block: extended bounds); first strip starts MR before it
-    const int jA = (R.j0 & ~1) - G::MR + strip * G::OW + 2 * lane;
+    // neighbour block: extended bounds); first strip starts MR before it.
+    // Shared edges: a CTA's warps march adjacent strips, the CTA loses MR columns per side.
+    const int jA = (kTbShare ? (R.j0 & ~1) - G::MR
+                             : (R.j0 & (TEA_TB_GEOM == 2 ? ~3 : ~1)) - G::SH) +
+                   (kTbShare ? blockIdx.x * G::OWC + warp * kStrip
+                             : (blockIdx.x * kTbW + warp) * G::OW) + 2 * lane;
+    const bool west_nb = kTbShare && warp > 0, east_nb = kTbShare && warp < kTbW - 1;
+    const int c_lo = west_nb ? 0 : (kTbShare ? G::MR : G::SH);
+    const int c_hi = east_nb ? kStrip : (kTbShare ? kStrip - G::MR : G::SH + G::OW);
     const int kt0 = R.k0 + blockIdx.y * ty;
     const int kt1 = min(kt0 + ty, R.k1);
     const int pitch = a.pitch;
     const bool ld_ok = jA + 1 < jlim;  // inside the allocation
     // output columns: this strip's [MR, 64-MR) intersected with the region
     const int cA = 2 * lane, cB = 2 * lane + 1;
-    const bool oA = cA >= G::MR && cA < kStrip - G::MR && jA >= R.j0 && jA < R.j1;
-    const bool oB = cB >= G::MR && cB < kStrip - G::MR && jA + 1 >= R.j0 && jA + 1 < R.j1;
+    const bool oA = cA >= c_lo && cA < c_hi && jA >= R.j0 && jA < R.j1;
+    const bool oB = cB >= c_lo && cB < c_hi && jA + 1 >= R.j0 && jA + 1 < R.j1;
     // dot products over owned cells only (D), whatever the extension of R
     const bool dA = oA && jA >= Dd.j0 && jA < Dd.j1, dB = oB && jA + 1 >= Dd.j0 && jA + 1 < Dd.j1;
 
@@ -361,6 +394,16 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     double2 W[M][3];
 #pragma unroll
     for (int t = 0; t < M; ++t) W[t][0] = W[t][1] = W[t][2] = z0;
+    // Shared strip edges, double-buffered by row parity: per warp and level t' < M the
+    // value row it produced this row-iteration -- lane 31's .y (the east warp's lane 0 west
+    // neighbour) and lane 0's Kx.x * value.x (the west warp's lane 31 east term) -- and
+    // lane 0's input-row Kx.x (the east face of the west warp's lane 31 cell B in diag(A)).
+    constexpr int NP = 2 * M + 1;
+    __shared__ double pub[2][kTbW][NP];
+    if (kTbShare) {
+        for (int i = threadIdx.x; i < 2 * kTbW * NP; i += kTbT) (&pub[0][0][0])[i] = 0.0;
+        __syncthreads();
+    }
     double dot0 = 0.0, dot1 = 0.0;
 
     const int kbeg = kt0 - M, kend = kt1 + M;
@@ -387,6 +430,9 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             }
             cp16(&cpa[sl][3][threadIdx.x], Kx + o);
             if (!KG) cp16(&cpa[sl][4][threadIdx.x], Ky + o);
+            // shared edges: lane 0 needs g(jA-1) for its west face (the west lane is in
+            // another warp) -- the 16-B pair g(jA-2), g(jA-1) into the free Ky slot
+            if (KG && kTbShare && lane == 0) cp16(&cpa[sl][4][threadIdx.x], Kx + o - 2);
         }
         cp_commit();  // one group per row, empty or not, so wait_group counts rows
     };
@@ -411,7 +457,8 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         double2 KX, KY;
         if (KG) {
             const double2 g = cpa[cs][3][threadIdx.x];
-            const double gW = __shfl_up_sync(0xffffffffu, g.y, 1);
+            double gW = __shfl_up_sync(0xffffffffu, g.y, 1);
+            if (kTbShare && lane == 0) gW = cpa[cs][4][threadIdx.x].y;
             // __dmul_rn: never contracted into an FMA with the faces' uses (the diagonal
             // sum below), so every face equals the stored one bit for bit
             KX.x = __dmul_rn(hrx, gW + g.x);
@@ -462,7 +509,9 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         // per row here, not once per step, and joins the row's slot (columns 12-15).
         // Kx(jA+2) (the face east of cell B) is the east lane's Kx(jA): one shuffle per row
         // (lane 31's value only feeds the margin).
-        const double kxE = __shfl_down_sync(0xffffffffu, s_kx.x, 1);
+        double kxE = __shfl_down_sync(0xffffffffu, s_kx.x, 1);
+        const int pb = (k - 1) & 1, cb = k & 1;  // parity buffers: previous row's, this row's
+        if (east_nb && lane == 31) kxE = pub[pb][warp + 1][2 * M];  // east warp's Kx(jA+2)
         double2 s_d;
         s_d.x = 1.0 + (s_kx.x + s_kx.y) + (s_ky.x + KY.x);
         s_d.y = 1.0 + (s_kx.y + kxE) + (s_ky.y + KY.y);
@@ -473,6 +522,13 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         W[0][0] = W[0][1];
         W[0][1] = W[0][2];
         W[0][2] = X;
+        if (kTbShare) {
+            if (lane == 0) {
+                pub[cb][warp][0] = KX.x * X.x;
+                pub[cb][warp][2 * M] = KX.x;
+            }
+            if (lane == 31) pub[cb][warp][1] = X.y;
+        }
 #pragma unroll
         for (int t = 1; t <= M; ++t) {
             const int q = k - t;
@@ -506,8 +562,10 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             // The per-step coefficients only ever multiply vector registers (uniform
             // operands, nothing hoisted into vector registers).
             const double2 dg = s_d;
-            const double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
-            const double east = __shfl_down_sync(0xffffffffu, kx.x * xc.x, 1);
+            double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
+            double east = __shfl_down_sync(0xffffffffu, kx.x * xc.x, 1);
+            if (west_nb && lane == 0) left = pub[pb][warp - 1][2 * (t - 1) + 1];
+            if (east_nb && lane == 31) east = pub[pb][warp + 1][2 * (t - 1)];
             double2 base, nb;
             base.x = cx * xc.x;
             base.y = cx * xc.y;
@@ -545,6 +603,10 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                 W[tt][0] = W[tt][1];
                 W[tt][1] = W[tt][2];
                 W[tt][2] = zn;
+                if (kTbShare) {
+                    if (lane == 0) pub[cb][warp][2 * tt] = kx.x * zn.x;
+                    if (lane == 31) pub[cb][warp][2 * tt + 1] = zn.y;
+                }
                 if (t == M - 1 && !LAST && rowout) st2m(zoutA + (orow - t * pitch), zn, oA, oB);
             } else {
                 if (rowout) {
@@ -572,6 +634,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
 #endif
             }
         }
+        if (kTbShare) __syncthreads();  // this row's edges published before the next row
     }
     asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory");
     __syncthreads();
@@ -598,9 +661,11 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     trace_end(a);
 }
 
+// output columns of one CTA of an M-step pass
 int tb_out_cols(int M) {
     const int mr = (M + 1) & ~1;
-    return kStrip - 2 * mr;
+    const int ow = TEA_TB_GEOM == 0 ? kStrip - 2 * M : (TEA_TB_GEOM == 2 ? 48 : kStrip - 2 * mr);
+    return kTbShare ? kTbW * kStrip - 2 * mr : kTbW * ow;
 }
 
 template <int M, bool FIRST, bool FUSE, bool LAST, bool KG>
@@ -611,8 +676,7 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
                       const double *ky, cudaStream_t st) {
     using G = TbGeom<M>;
     const int width = R.j1 - (R.j0 & ~1);
-    const int nstrips = (width + G::OW - 1) / G::OW;
-    dim3 grid((nstrips + kTbW - 1) / kTbW, (R.k1 - R.k0 + ty - 1) / ty);
+    dim3 grid((width + G::OWC - 1) / G::OWC, (R.k1 - R.k0 + ty - 1) / ty);
     constexpr size_t smem = tb_smem_bytes();
     // > 48 KB of dynamic shared memory needs the attribute, set once per device
     static std::atomic<unsigned long long> attr{0ull};  // per instantiation: device bit mask
@@ -687,7 +751,7 @@ int tb_auto_rows(int M, int width, int height) {
     int slots[8] = {};
     slots[M] = slots_m;
     const int ow = tb_out_cols(M);
-    const int gx = ((width + ow - 1) / ow + kTbW - 1) / kTbW;
+    const int gx = (width + ow - 1) / ow;
     int best = height, bestc = 0x7fffffff;
     for (int w = 1; w <= 256; ++w) {
         const int tiles = (int)((long long)slots[M] * w / gx);
@@ -706,8 +770,7 @@ int tb_auto_rows(int M, int width, int height) {
 
 int tb_ctas(int M, int width, int height, int ty) {
     const int ow = tb_out_cols(M);
-    const int nstrips = (width + ow - 1) / ow;
-    return ((nstrips + kTbW - 1) / kTbW) * ((height + ty - 1) / ty);
+    return ((width + ow - 1) / ow) * ((height + ty - 1) / ty);
 }
 
 void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, int ty, int jlim,

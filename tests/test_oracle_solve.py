@@ -214,28 +214,31 @@ def test_cg1_conservation(ora):
 # ---------------------------------------------------------------- single-reduction CPPCG
 @pytest.mark.parametrize("kind,nx,ny,seed,dt", SMALL)
 @pytest.mark.parametrize("s", [4, 10])
-def test_cppcg1_dense_direct_solve(ora, kind, nx, ny, seed, dt, s):
+@pytest.mark.parametrize("fused", [False, True])
+def test_cppcg1_dense_direct_solve(ora, kind, nx, ny, seed, dt, s, fused):
     """Chronopoulos-Gear PCG with M^{-1} = B(A) (NEXT-2 for CPPCG) reaches the
-    dense solution."""
+    dense solution: s = A p by recurrence (CPPCG1) and w = A p applied (CPPCG1F, R23)."""
     d = (inputs.random_fields(nx, ny, seed, dt=dt) if kind == "random"
          else inputs.crooked_pipe(nx, ny))
     Kx, Ky, u0 = setup(ora, d)
     ustar = np.linalg.solve(dense_A(ora, Kx, Ky, nx, ny), u0.ravel()).reshape(ny, nx)
-    res = ora.solve(Kx, Ky, u0, method=ora.CPPCG1, eps=1e-15, max_iters=5000, inner_steps=s,
-                    presteps=8)
+    res = ora.solve(Kx, Ky, u0, method=ora.CPPCG1F if fused else ora.CPPCG1, eps=1e-15,
+                    max_iters=5000, inner_steps=s, presteps=8)
     assert res.status == 0
     assert np.abs(res.u - ustar).max() / np.abs(ustar).max() <= 1e-11
 
 
 @pytest.mark.parametrize("n,s", [(64, 10), (128, 10), (96, 5)])
-def test_cppcg1_equivalent_to_cppcg(ora, n, s):
+@pytest.mark.parametrize("fused", [False, True])
+def test_cppcg1_equivalent_to_cppcg(ora, n, s, fused):
     """Same Krylov iterates as CPPCG in exact arithmetic: the same presteps and
     eigen-estimate, outer iteration counts within +-2, fields equal, and the same
     residual norm and iterate after every fixed outer count (to rounding)."""
     d = inputs.crooked_pipe(n)
     Kx, Ky, u0 = setup(ora, d)
+    m1 = ora.CPPCG1F if fused else ora.CPPCG1
     a = ora.solve(Kx, Ky, u0, method=ora.CPPCG, eps=1e-13, max_iters=100000, inner_steps=s)
-    b = ora.solve(Kx, Ky, u0, method=ora.CPPCG1, eps=1e-13, max_iters=100000, inner_steps=s)
+    b = ora.solve(Kx, Ky, u0, method=m1, eps=1e-13, max_iters=100000, inner_steps=s)
     assert a.status == b.status == 0
     assert a.stats["presteps"] == b.stats["presteps"] == 30
     assert a.stats["eig_max"] == b.stats["eig_max"]
@@ -243,22 +246,38 @@ def test_cppcg1_equivalent_to_cppcg(ora, n, s):
     assert np.abs(a.u - b.u).max() / np.abs(a.u).max() <= 1e-11
     for k in (1, 3, 8):
         x = ora.solve(Kx, Ky, u0, method=ora.CPPCG, eps=0.0, max_iters=30 + k, inner_steps=s)
-        y = ora.solve(Kx, Ky, u0, method=ora.CPPCG1, eps=0.0, max_iters=30 + k, inner_steps=s)
+        y = ora.solve(Kx, Ky, u0, method=m1, eps=0.0, max_iters=30 + k, inner_steps=s)
         assert x.stats["outer"] == y.stats["outer"] == k
         assert y.stats["rnorm"] == pytest.approx(x.stats["rnorm"], rel=1e-8)
         assert np.abs(x.u - y.u).max() / np.abs(x.u).max() <= 1e-12
     # matvec accounting: residual + 30 presteps + the restart's s inner steps, then per
     # outer iteration s inner steps + one matvec (CPPCG: A p; CPPCG1: q = A z, plus one at
-    # the restart)
+    # the restart; CPPCG1F: A p and q = A z, plus one at the restart)
     assert a.stats["matvecs"] == 1 + 30 + s + a.stats["outer"] * (s + 1)
-    assert b.stats["matvecs"] == 1 + 30 + s + 1 + b.stats["outer"] * (s + 1)
+    assert b.stats["matvecs"] == 1 + 30 + s + 1 + b.stats["outer"] * (s + (2 if fused else 1))
 
 
-def test_cppcg1_conservation_and_limits(ora):
+@pytest.mark.parametrize("n,s", [(64, 10), (96, 5)])
+def test_cppcg1f_equals_cppcg1_recurrence(ora, n, s):
+    """The two single-reduction forms share their scalars (gam, del, alpha, beta) and differ
+    only in how A p enters r: applied (CPPCG1F) or by the recurrence s = q + beta s (CPPCG1);
+    the iterates agree to rounding after every fixed outer count."""
+    d = inputs.crooked_pipe(n)
+    Kx, Ky, u0 = setup(ora, d)
+    for k in (1, 2, 5):
+        x = ora.solve(Kx, Ky, u0, method=ora.CPPCG1, eps=0.0, max_iters=30 + k, inner_steps=s)
+        y = ora.solve(Kx, Ky, u0, method=ora.CPPCG1F, eps=0.0, max_iters=30 + k, inner_steps=s)
+        assert y.stats["rnorm"] == pytest.approx(x.stats["rnorm"], rel=1e-8)
+        assert np.abs(x.u - y.u).max() / np.abs(x.u).max() <= 1e-12
+
+
+@pytest.mark.parametrize("fused", [False, True])
+def test_cppcg1_conservation_and_limits(ora, fused):
     d = inputs.crooked_pipe(48)
     Kx, Ky, u0 = setup(ora, d)
+    m1 = ora.CPPCG1F if fused else ora.CPPCG1
     for k in (31, 33, 40):
-        res = ora.solve(Kx, Ky, u0, method=ora.CPPCG1, eps=0.0, max_iters=k, inner_steps=6)
+        res = ora.solve(Kx, Ky, u0, method=m1, eps=0.0, max_iters=k, inner_steps=6)
         assert res.status == 1 and res.stats["iterations"] == k
         assert abs(res.u.sum() - u0.sum()) / u0.sum() <= 1e-13
-    assert ora.solve(Kx, Ky, u0, method=ora.CPPCG1, inner_steps=0).status == -1
+    assert ora.solve(Kx, Ky, u0, method=m1, inner_steps=0).status == -1
