@@ -173,7 +173,7 @@ def cpu_info():
 
 
 # ------------------------------------------------------------------ oracle timing
-TWO_PHASE = ("cppcg", "cppcg1", "cheby")
+TWO_PHASE = ("cppcg", "cppcg1", "cppcg1f", "cheby")
 # iteration mix of one timestep of the headline workload on the GPU (4096^2 pipe CPPCG s=10,
 # eps 1e-12, timesteps 6-25 of the bench: 30 presteps + 253.1 outer, profiles/r01j_bench.json;
 # the oracle's counts agree within +-2, tests/test_gpu_parity.py): used by the reference arm,
@@ -190,7 +190,7 @@ def oracle_phase_costs(args, deck):
     oracle.build()
     method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
               "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY,
-              "cppcg1": oracle.CPPCG1}[args.method]
+              "cppcg1": oracle.CPPCG1, "cppcg1f": oracle.CPPCG1F}[args.method]
     if args.nz > 1:
         rx, ry, rz = oracle.mesh_r3(deck)
         K = oracle.face_coefficients3(deck.nx, deck.ny, deck.nz, rx, ry, rz, deck.density)
@@ -248,7 +248,7 @@ def run_reference(args):
     deck = make_deck(args)
     method = {"cppcg": oracle.CPPCG, "cg": oracle.CG, "bjcg": oracle.BJCG,
               "cg1": oracle.CG1, "jacobi": oracle.JACOBI, "cheby": oracle.CHEBY,
-              "cppcg1": oracle.CPPCG1}[args.method]
+              "cppcg1": oracle.CPPCG1, "cppcg1f": oracle.CPPCG1F}[args.method]
     orun = oracle.run3 if args.nz > 1 else oracle.run
     costs = oracle_phase_costs(args, deck)  # (part of the warm-up)
     two = "t_pre" in costs
@@ -299,7 +299,8 @@ def run_reference(args):
 
 METHOD_NAME = {"cppcg": "CPPCG", "cg": "CG", "bjcg": "block-Jacobi PCG",
                "cg1": "single-reduction CG", "jacobi": "Jacobi", "cheby": "Chebyshev",
-               "cppcg1": "single-reduction CPPCG"}
+               "cppcg1": "single-reduction CPPCG",
+               "cppcg1f": "single-reduction CPPCG (fused form)"}
 
 
 def make_deck(args):
@@ -408,7 +409,7 @@ def run_gpu(args):
     deck = make_deck(args)
     method = {"cppcg": tea.CPPCG, "cg": tea.CG, "bjcg": tea.BJCG,
               "cg1": tea.CG1, "jacobi": tea.JACOBI, "cheby": tea.CHEBY,
-              "cppcg1": tea.CPPCG1}[args.method]
+              "cppcg1": tea.CPPCG1, "cppcg1f": tea.CPPCG1F}[args.method]
     cells = args.n * args.n * max(args.nz, 1)
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
                 tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode,
@@ -554,7 +555,7 @@ def main():
     ap.add_argument("--nz", type=int, default=0,
                     help="> 1: the 3D 7-point problem on n x n x nz (SURVEY NEXT-4)")
     ap.add_argument("--method", default="cppcg", choices=["cppcg", "cg", "bjcg", "cg1", "jacobi", "cheby",
-                                                   "cppcg1"])
+                                                   "cppcg1", "cppcg1f"])
     ap.add_argument("--inner", type=int, default=10)
     ap.add_argument("--eps", type=float, default=1e-12)
     ap.add_argument("--max-iters", type=int, default=0,
@@ -588,7 +589,7 @@ def main():
     if args.warmup < 3:
         ap.error("--warmup must be >= 3")
     if args.halo_depth == 0:
-        args.halo_depth = args.inner + 1 if args.method in ("cppcg", "cppcg1") else 1
+        args.halo_depth = args.inner + 1 if args.method in ("cppcg", "cppcg1", "cppcg1f") else 1
     if args.max_iters == 0:
         args.max_iters = 2000 if args.method in ("jacobi", "cheby") else 100000
     if args.impl == "reference":

@@ -64,9 +64,17 @@ typedef enum {
  * (as CPPCG). One stencil pass per iteration; the stop test uses the true residual of
  * the iterate before the last update (reading R19). Chebyshev "cannot cope with some
  * condition numbers": max_iters bounds it.                          */
+/* TEA_CPPCG1F: single-reduction CPPCG in fused form (reading R23): the scalars of TEA_CPPCG1
+ * (one reduction of z.q, r.z, r.r per outer iteration) with w = A p applied
+ * instead of carried by recurrence. On one block with the fused passes an outer iteration is
+ * TWO kernels: the first pass does the outer update (p = z + beta p, u += alpha p,
+ * r -= alpha A p) and the first Chebyshev steps, the last pass the last steps and q = A z
+ * with the three dot products -- 15 fp64 streams (TEA_CPPCG: 3 kernels, 18 streams; TEA_CPPCG1:
+ * 4 kernels, 22). Same iterates as CPPCG in exact arithmetic; s + 2 matvecs per outer
+ * iteration. 2D.                                                                     */
 typedef enum {
     TEA_CG = 0, TEA_CPPCG = 1, TEA_BJCG = 2, TEA_CG1 = 3, TEA_JACOBI = 4, TEA_CHEBY = 5,
-    TEA_CPPCG1 = 6
+    TEA_CPPCG1 = 6, TEA_CPPCG1F = 7
 } tea_method;
 
 typedef struct tea_ctx tea_ctx; /* opaque, library-owned */

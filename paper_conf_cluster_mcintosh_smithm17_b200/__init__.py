@@ -20,7 +20,7 @@ import numpy as np
 
 from . import _build
 
-CG, CPPCG, BJCG, CG1, JACOBI, CHEBY, CPPCG1 = 0, 1, 2, 3, 4, 5, 6
+CG, CPPCG, BJCG, CG1, JACOBI, CHEBY, CPPCG1, CPPCG1F = 0, 1, 2, 3, 4, 5, 6, 7
 OK, NOT_CONVERGED = 0, 1
 ERR_ARG, ERR_CUDA, ERR_NCCL, ERR_BREAKDOWN, ERR_STATE = -1, -2, -3, -4, -5
 KERNELS = ["init", "residual", "spmv", "update", "cheb_first", "cheb_step", "cheb_last", "eig",

@@ -619,6 +619,28 @@ int tb_steps(const tea_ctx *c) {
 bool single_block(tea_ctx *c) { return c->px * c->py == 1; }
 bool is3d(const tea_ctx *c) { return c->blocks[0].L.nz > 1; }
 
+// Extra work of a temporally blocked chain (single-reduction CPPCG in fused form, CPPCG1F):
+// pre = the first pass starts with the outer update p = z_s + beta p, u += alpha p,
+// r' = r - alpha A p (reads z_s, p_in, r, u; writes p_out, u, r'); post = the last pass ends
+// with q = A z_s and z_s . q (a third value in its grid reduction).
+struct ChainX {
+    bool pre = false, post = false;
+    bool even = false;  // CPPCG1F on one block: the pass split of chain_passes(.., true)
+    int zs = -1, pin = -1, pout = -1;
+};
+
+// Passes of a chain. CPPCG1F on one block (pre and post): an even number of passes >= 2, so
+// the first pass's output pair never aliases the z_s it reads (the last pass's pair).
+std::vector<int> chain_passes(const tea_ctx *c, int s, bool f1) {
+    if (!f1) return tb_passes(s, tb_steps(c));
+    const int mmax = std::min(tb_steps(c), kTbMaxSteps);
+    int P = std::max(2, (s + mmax - 1) / mmax);
+    if (P % 2) ++P;
+    std::vector<int> v;
+    for (int p = 0; p < P; ++p) v.push_back(s / P + (p < s % P ? 1 : 0));
+    return v;
+}
+
 // Temporally blocked chain: passes of M steps, each ONE kernel per block
 // (tea_cheb_tb.cu). z pairs ping-pong: pass p writes (z_{last-1}, z_last) into
 // pair p%2 = (Z0,Z1) or (Z2,Z3). Returns the field holding z_s.
@@ -627,8 +649,9 @@ bool is3d(const tea_ctx *c) { return c->blocks[0].L.nz > 1; }
 // 1 + (steps after it), so the last pass leaves z_s valid on the 1-cell ring the next
 // SpMV reads; no z exchange. (One block: every extension is empty.)
 int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout,
-                  bool sets_cond, bool reduce_dots = true) {
-    const auto passes = tb_passes(s, tb_steps(c));
+                  bool sets_cond, bool reduce_dots = true, const ChainX &x = ChainX()) {
+    const bool f1 = x.pre;  // CPPCG1F's one-block fused outer update
+    const auto passes = chain_passes(c, s, x.even);
     const int pairA[2] = {F_Z0, F_Z2}, pairB[2] = {F_Z1, F_Z3};
     const bool blocks = !single_block(c);
     // Overlap: the depth-d exchange of r runs on the exchange stream while
@@ -649,12 +672,14 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
         }
     }
     int step0 = 1, after = s;
-    const int r = fused ? rout : rin;
+    const int r = (fused || f1) ? rout : rin;
     for (size_t p = 0; p < passes.size(); ++p) {
         const int M = passes[p];
         after -= M;
         const bool first = p == 0, last = p + 1 == passes.size();
         const bool fu = fused && first;
+        const bool pre = x.pre && first, post = x.post && last;
+        const int levels = M + (pre ? 1 : 0) + (post ? 1 : 0);
         const int o = p % 2, in = (p + 1) % 2;
         // the regions this pass is launched on, per block: the whole (extended) region, or
         // for the overlapped first pass the halo-free interior now and the frame after the
@@ -695,27 +720,45 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
             const Region D = b.owned();
             const int jlim = b.L.pitch - b.L.X0;
             int ty = c->opts.tb_rows > 0 ? c->opts.tb_rows : 0;
-            // tall tiles keep the 2M-row pipeline fill small; whole waves (tb_auto_rows)
-            if (ty <= 0) ty = tb_auto_rows(M, R.j1 - R.j0, R.k1 - R.k0);
-            // two reduction partials per CTA must fit the block's scratch
+            // tall tiles keep the 2-level-row pipeline fill small; whole waves (tb_auto_rows)
+            if (ty <= 0) ty = tb_auto_rows(levels, R.j1 - R.j0, R.k1 - R.k0);
+            // the reduction partials (2 or 3 per CTA) must fit the block's scratch
+            const size_t nv = post ? 3 : 2;
             while (ty < R.k1 - R.k0 &&
-                   2 * (size_t)tb_ctas(M, R.j1 - R.j0, R.k1 - R.k0, ty) > b.L.partials_cap)
+                   nv * (size_t)tb_ctas(levels, R.j1 - R.j0, R.k1 - R.k0, ty) > b.L.partials_cap)
                 ty *= 2;
-            int streams = (first ? (fu ? 2 : 1) : 3) + kstreams(c, b);  // reads
-            streams += (fu ? 1 : 0) + (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})
+            // algorithmic streams: reads, then writes
+            int streams;
+            if (pre)
+                streams = 4 + kstreams(c, b) + 3 + (last ? 1 : 2);  // z_s, p, r, u, g -> p, u, r', z..
+            else
+                streams = (first ? (fu ? 2 : 1) : 3) + kstreams(c, b) + (fu ? 1 : 0) +
+                          (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})
             const int kid = last ? TEA_K_TB_LAST : (first ? TEA_K_TB_FIRST : TEA_K_TB_MID);
+            TbArgs f;
+            f.rin = b.f[first && (fu || pre) ? rin : r];
+            f.win = b.f[F_W];
+            f.rout = b.f[rout];
+            f.zin1 = pre ? b.f[x.zs] : (first ? nullptr : b.f[pairB[in]]);
+            f.zin2 = first ? nullptr : b.f[pairA[in]];
+            f.zoutA = b.f[pairA[o]];
+            f.zoutB = b.f[pairB[o]];
+            f.kx = b.f[F_KX];
+            f.ky = b.f[F_KY];
+            if (pre) {
+                f.pin = b.f[x.pin];
+                f.pout = b.f[x.pout];
+                f.uio = b.f[F_U];
+            }
             K(c, kid, sbytes(b, streams), [&] {
                 launch_cheb_tb(kargs(c, b, last && sets_cond), R, D, M, ty, jlim, step0, first,
-                               fu, last, restart, b.f[first && fu ? rin : r], b.f[F_W],
-                               b.f[rout], first ? nullptr : b.f[pairB[in]],
-                               first ? nullptr : b.f[pairA[in]], b.f[pairA[o]], b.f[pairB[o]],
-                               b.f[F_KX], b.f[F_KY], c->stream);
+                               fu, last, restart, pre, post, f, c->stream);
             });
           }
         }
         step0 += M;
     }
-    if (reduce_dots) reduce(c, 1, 2);
+    if (reduce_dots) reduce(c, x.post ? 0 : 1, x.post ? 3 : 2);
     return pairB[(passes.size() - 1) % 2];
 }
 
@@ -725,6 +768,10 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
 bool use_tb(tea_ctx *c, int s) {
     if (is3d(c) || tb_steps(c) <= 1 || c->coef_slot < 0) return false;
     return single_block(c) || c->d >= s + 1;
+}
+// CPPCG1F: the pre / post levels form faces from g (kform >= 0) and need >= 2 passes
+bool use_tb1f(tea_ctx *c, int s) {
+    return use_tb(c, s) && c->opts.kform >= 0 && (!single_block(c) || s >= 2);
 }
 
 // reduce_dots = false: the caller folds the chain's [r.z, r.r] into its own single
@@ -740,6 +787,14 @@ int chain(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout, bool s
 int zs_field(tea_ctx *c, int s) {
     if (use_tb(c, s)) {
         const int P = (int)tb_passes(s, tb_steps(c)).size();
+        return (P - 1) % 2 == 0 ? F_Z1 : F_Z3;
+    }
+    return zbuf(s);
+}
+// ... of CPPCG1F's chains: one block fused -> an even pass count -> Z3
+int zs_field1f(tea_ctx *c, int s) {
+    if (use_tb1f(c, s)) {
+        const int P = (int)chain_passes(c, s, single_block(c)).size();
         return (P - 1) % 2 == 0 ? F_Z1 : F_Z3;
     }
     return zbuf(s);
@@ -842,6 +897,53 @@ void body_pcg1(tea_ctx *c, int s, int /*par*/, bool sets_cond) {
             launch_cg1_update(kargs(c, b), L, R, b.f[F_W], b.f[F_R1], b.f[F_P0], b.f[F_U],
                               b.f[F_R0], c->stream, b.f[zs]);
         });
+    }
+    chain(c, s, false, false, F_R0, F_R0, false, false);
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan_st(c, b, R);
+        K(c, TEA_K_CG1W, sbytes(b, 2 + kstreams(c, b)), [&] {
+            launch_cg1_w(kargs(c, b, sets_cond), L, R, b.f[zs], b.f[F_W], b.f[F_KX], b.f[F_KY],
+                         c->stream, true);
+        });
+    }
+    reduce(c, 0, 3);
+}
+
+// Single-reduction CPPCG in fused form (CPPCG1F; oracle ORA_CPPCG1F, reading R23): ONE
+// reduction of [z.q, r.z, r.r] per outer iteration, like CPPCG1, with A p applied instead of
+// carried. One block with the fused passes: TWO kernels per outer iteration -- the first pass
+// does the outer update (p = z_s + beta p, u += alpha p, r' = r - alpha A p) and the first
+// Chebyshev steps, the last pass the last steps and q = A z_s with the three dots (15 streams:
+// 5 reads + 5 writes, then 4 + 1; CPPCG: 3 kernels, 18 streams). Blocks / one kernel per
+// step: the update as one stencil pass (k_cg1f_pre), the chain (with the post level on the
+// fused path, else q = A z_s by k_cg1_w), then the reduction.
+// Fields: z_s in zs_field1f, p ping-pong P0/P1 by par; r ping-pong R0/R1 by par on the one-block
+// fused path, in place (R0) otherwise.
+void body_pcg1f(tea_ctx *c, int s, int par, bool sets_cond) {
+    const int zs = zs_field1f(c, s);
+    if (single_block(c) && use_tb1f(c, s)) {
+        ChainX x;
+        x.pre = x.post = x.even = true;
+        x.zs = zs;
+        x.pin = F_P0 + par;
+        x.pout = F_P1 - par;
+        cheb_chain_tb(c, s, false, false, F_R0 + par, F_R1 - par, sets_cond, true, x);
+        return;
+    }
+    for (auto &b : c->blocks) {
+        Region R = b.owned();
+        Launch L = plan_spmv(c, b, R);
+        K(c, TEA_K_UPDATE, sbytes(b, 7 + kstreams(c, b)), [&] {  // z, p, r, u -> p, r, u
+            launch_cg1f_pre(kargs(c, b), L, R, b.f[zs], b.f[F_P0 + par], b.f[F_P1 - par],
+                            b.f[F_R0], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
+        });
+    }
+    if (use_tb1f(c, s)) {
+        ChainX x;
+        x.post = true;
+        cheb_chain_tb(c, s, false, false, F_R0, F_R0, sets_cond, true, x);
+        return;
     }
     chain(c, s, false, false, F_R0, F_R0, false, false);
     for (auto &b : c->blocks) {
@@ -1024,10 +1126,10 @@ void solve_persist(tea_ctx *c, int s, bool two_phase) {
 tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, int s,
                       tea_stats *st) {
     if (c->failed) fail(TEA_ERR_STATE, "context already failed: %s", c->err.c_str());
-    if (method < TEA_CG || method > TEA_CPPCG1) fail(TEA_ERR_ARG, "bad method %d", (int)method);
+    if (method < TEA_CG || method > TEA_CPPCG1F) fail(TEA_ERR_ARG, "bad method %d", (int)method);
     if (method == TEA_BJCG && is3d(c)) fail(TEA_ERR_ARG, "block Jacobi is 2D only");
     if (max_iters < 0) fail(TEA_ERR_ARG, "max_iters < 0");
-    const bool pcg = method == TEA_CPPCG || method == TEA_CPPCG1;
+    const bool pcg = method == TEA_CPPCG || method == TEA_CPPCG1 || method == TEA_CPPCG1F;
     if (pcg && (s < 1 || s > kMaxS))
         fail(TEA_ERR_ARG, "inner_steps must be in [1,%d]", kMaxS);
     const int pre = c->opts.presteps;
@@ -1140,7 +1242,27 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         // the fused passes read the coefficients from constant memory (every block's copy
         // is identical: they derive from globally reduced scalars)
         if (use_tb(c, s)) CK(tb_coef_upload(c->coef_slot, c->blocks[0].S, c->stream));
-        if (method == TEA_CPPCG1) {
+        if (method == TEA_CPPCG1F) {
+            // z = B(A) r, q = A z, [z.q, r.z, r.r] in one reduction (b_0 = 0)
+            if (use_tb1f(c, s)) {
+                ChainX x;
+                x.post = true;
+                x.even = single_block(c);
+                cheb_chain_tb(c, s, true, false, F_R0, F_R0, false, true, x);
+            } else {
+                chain(c, s, true, false, F_R0, F_R0, false, false);
+                const int zs = zs_field1f(c, s);
+                for (auto &b : c->blocks) {
+                    Region R = b.owned();
+                    Launch L = plan_st(c, b, R);
+                    K(c, TEA_K_CG1W, sbytes(b, 2 + kstreams(c, b)), [&] {
+                        launch_cg1_w(kargs(c, b), L, R, b.f[zs], b.f[F_W], b.f[F_KX], b.f[F_KY],
+                                     c->stream, true);
+                    });
+                }
+                reduce(c, 0, 3);
+            }
+        } else if (method == TEA_CPPCG1) {
             // z = B(A) r, q = A z, [z.q, r.z, r.r] in one reduction; p = s = 0 (b_0 = 0)
             chain(c, s, true, false, F_R0, F_R0, false, false);
             const int zs = zs_field(c, s);
@@ -1161,6 +1283,9 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
             if (method == TEA_CPPCG1)
                 run_loop(c, 7 + 16LL * s, max_iters,
                          [&](int par, bool sc) { body_pcg1(c, s, par, sc); });
+            else if (method == TEA_CPPCG1F)
+                run_loop(c, 8 + 16LL * s, max_iters,
+                         [&](int par, bool sc) { body_pcg1f(c, s, par, sc); });
             else
                 run_loop(c, 2 + 16LL * s, max_iters,
                          [&](int par, bool sc) { body_pcg(c, s, par, sc); });
@@ -1183,7 +1308,8 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
         st->outer = phase2 ? h.outer : 0;
         st->inner_matvecs = phase2 && pcg ? s * (h.outer + 1) : 0;
         st->matvecs = 1 + h.it + st->inner_matvecs + (method == TEA_CG1 ? 1 : 0) +
-                      (phase2 && method == TEA_CPPCG1 ? 1 : 0);
+                      (phase2 && method == TEA_CPPCG1 ? 1 : 0) +
+                      (phase2 && method == TEA_CPPCG1F ? 1 + h.outer : 0);
         st->status = rs;
         st->r0 = h.r0;
         st->rnorm = std::sqrt(h.red_rr);

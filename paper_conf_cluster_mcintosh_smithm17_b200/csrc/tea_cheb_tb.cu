@@ -179,38 +179,37 @@ __device__ __forceinline__ double2 tm_get(const TmRow &o, int i) {
     return make_double2(d_of(o.v[4 * i], o.v[4 * i + 1]), d_of(o.v[4 * i + 2], o.v[4 * i + 3]));
 }
 
-// Deterministic two-value grid reduction (same scheme as tea_kernels.cu).
-__device__ bool grid_reduce2(double v0, double v1, double *partials, unsigned *ticket,
-                             double *out0, double *out1) {
-    __shared__ double sh[2][kTbW];
+// Deterministic NV-value grid reduction (same scheme as tea_kernels.cu): fixed-order warp,
+// CTA and partials sums; returns true in the last CTA, whose threads then hold the totals.
+template <int NV>
+__device__ bool grid_reduce_n(const double (&v)[NV], double *partials, unsigned *ticket,
+                              double (&out)[NV]) {
+    __shared__ double sh[NV][kTbW];
     __shared__ bool last;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const int nblk = gridDim.x * gridDim.y * gridDim.z;
     const int bid = (blockIdx.z * gridDim.y + blockIdx.y) * gridDim.x + blockIdx.x;
-    v0 = wsum(v0);
-    v1 = wsum(v1);
-    if (lane == 0) {
-        sh[0][warp] = v0;
-        sh[1][warp] = v1;
+#pragma unroll
+    for (int i = 0; i < NV; ++i) {
+        const double w = wsum(v[i]);
+        if (lane == 0) sh[i][warp] = w;
     }
     __syncthreads();
     if (threadIdx.x == 0) {
-        double s0 = 0.0, s1 = 0.0;
-        for (int w = 0; w < kTbW; ++w) {
-            s0 += sh[0][w];
-            s1 += sh[1][w];
+#pragma unroll
+        for (int i = 0; i < NV; ++i) {
+            double s0 = 0.0;
+            for (int w = 0; w < kTbW; ++w) s0 += sh[i][w];
+            partials[i * nblk + bid] = s0;
         }
-        partials[bid] = s0;
-        partials[nblk + bid] = s1;
         __threadfence();
         last = (atomicAdd(ticket, 1u) == (unsigned)nblk - 1u);
     }
     __syncthreads();
     if (!last) return false;
     __threadfence();
-    double t[2];
 #pragma unroll
-    for (int i = 0; i < 2; ++i) {
+    for (int i = 0; i < NV; ++i) {
         double s = 0.0;
         for (int b = threadIdx.x; b < nblk; b += kTbT) s += __ldcg(partials + i * nblk + b);
         s = wsum(s);
@@ -219,10 +218,8 @@ __device__ bool grid_reduce2(double v0, double v1, double *partials, unsigned *t
         __syncthreads();
         double a = 0.0;
         for (int w = 0; w < kTbW; ++w) a += sh[i][w];
-        t[i] = a;
+        out[i] = a;
     }
-    *out0 = t[0];
-    *out1 = t[1];
     if (threadIdx.x == 0) *ticket = 0u;
     return true;
 }
@@ -250,9 +247,6 @@ __device__ bool grid_arrive2(unsigned *ticket) {
 #ifndef TEA_TB_CPA_L
 #define TEA_TB_CPA_L 2
 #endif
-#ifndef TEA_TB_DIAG
-#define TEA_TB_DIAG 1
-#endif
 // Row-loop unroll and cp.async depth of the first pass (carries r, w and the update) and of
 // the later passes, measured separately (profiles/r01g_tmem_cpa.txt): unrolling by the
 // window period 3 turns the W[t][*] rotation into register renaming instead of ~50 moves per
@@ -269,37 +263,25 @@ constexpr size_t tb_smem_bytes() {
                : 48u * 1024u;
 }
 
-#ifndef TEA_TB_SHARE
-#define TEA_TB_SHARE 0
-#endif
-// TEA_TB_SHARE (measured, not kept -- DESIGN.md §4.4): the warps of a CTA march adjacent
-// 64-column strips and hand each other their strip-edge values through shared memory once per
-// row (one CTA barrier per row), so a CTA loses MR columns per side instead of every warp
-// (244 of 256 columns at M = 5 instead of 4 x 54). Bitwise the same results, but the barrier
-// couples the 4 warps' latency chains: 274 vs 179 us per pass at 4096^2
-// (profiles/r02_tb_share_ab.txt).
-constexpr bool kTbShare = TEA_TB_SHARE != 0;
-// Strip geometry (unshared): a warp's 64 columns output [SH, SH + OW); strips start SH
-// before the region at a stride of OW. 1 (default): SH = MR = M rounded up to even,
-// OW = 64 - 2 MR (52 at M = 5). 0: OW = 64 - 2M (54 at M = 5: fewer redundant columns but
-// 215 vs 184 us per first pass at 4096^2 -- strip starts at 8 offsets mod 128 B instead of 4,
-// profiles/r02_knobs_ab.txt). 2: SH = 8, OW = 48 (M <= 8): every strip starts on a 32-B
-// sector, x1.33 redundant work.
+// Strip geometry: a warp's 64 columns output [SH, SH + OW); strips start SH before the
+// region at a stride of OW. 1 (default): SH = MR = levels rounded up to even, OW = 64 - 2 MR
+// (52 at 5 levels). 0: OW = 64 - 2 levels (54 at 5 levels: fewer redundant columns but 215 vs
+// 184 us per first pass at 4096^2 -- strip starts at 8 offsets mod 128 B instead of 4,
+// profiles/r02_knobs_ab.txt). 2: SH = 8, OW = 48: every strip starts on a 32-B sector, x1.33
+// redundant work (slower). Sharing strip edges between the 4 warps of a CTA through shared
+// memory (one CTA barrier per row; 244 of 256 columns) was bitwise equal but 274 vs 179 us:
+// the barrier couples the warps' latency chains (profiles/r02_tb_share_ab.txt).
 #ifndef TEA_TB_GEOM
 #define TEA_TB_GEOM 1
 #endif
-template <int M>
+template <int NL>  // NL = stencil levels of the pass
 struct TbGeom {
-    static constexpr int MR = (M + 1) & ~1;  // first strip's shift: >= M, even (double2 loads)
-    // output columns per warp strip (unshared): [M, 64 - M) -- the stride 64 - 2M is even, so
-    // every strip still starts on a double2 (M = 5: 54 columns, x1.185 redundant work)
+    static constexpr int MR = (NL + 1) & ~1;  // >= NL, even (double2 loads)
     static constexpr int SH = TEA_TB_GEOM == 2 ? 8 : MR;
-    static constexpr int OW = TEA_TB_GEOM == 0 ? kStrip - 2 * M
+    static constexpr int OW = TEA_TB_GEOM == 0 ? kStrip - 2 * NL
                               : (TEA_TB_GEOM == 2 ? 48 : kStrip - 2 * MR);
-    static_assert(SH >= M && SH + OW <= kStrip - M && OW % 2 == 0, "strip geometry");
-    // output columns per CTA
-    static constexpr int OWC = kTbShare ? kTbW * kStrip - 2 * MR : kTbW * OW;
-    static constexpr int D = 8;  // TMEM ring depth (rows k-M-1..k fit for M <= 6); a power of
+    static_assert(SH >= NL && SH + OW <= kStrip - NL && OW % 2 == 0, "strip geometry");
+    static constexpr int D = 8;  // TMEM ring depth (rows k-NL..k fit for NL <= 6); a power of
                                  // two so slots are (head - t) & 7
 };
 
@@ -312,17 +294,30 @@ constexpr int kTmCols = 128;  // TMEM columns per 4 warps: 8 slots x 16 per warp
 // as it arrives -- Kx(j) = hrx (g(j-1) + g(j)) with g(j-1) from the west lane (lane 0's
 // west face is a margin column, polluted like its west operand), Ky(k) = hry (g(k-1) + g(k))
 // with g(k-1) the previous row's -- one staged stream instead of two, same faces bit for bit.
-template <int M, bool FIRST, bool FUSE, bool LAST, bool KG>
+//
+// PRE / POST (single-reduction CPPCG in fused form, TEA_CPPCG1F, oracle ORA_CPPCG1F, reading
+// R23): the first pass starts with the outer update -- level 0 forms p = z + beta p_old and
+// writes p and u += alpha p, level 1 applies A to p and forms r' = r - alpha (A p) (written,
+// and replacing r in the row's TMEM slot), then the M Chebyshev steps; the last pass ends with
+// one more stencil level q = A z_s whose z_s . q joins r.z and r.r in ONE grid reduction.
+// alpha and beta come from the previous reduction (Chronopoulos & Gear). Every level loses a
+// column per side and lags a row: NL = M + PRE + POST <= 6 levels.
+template <int M, bool FIRST, bool FUSE, bool LAST, bool KG, bool PRE, bool POST>
 __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     k_cheb_tb(const double *__restrict__ rin, const double *__restrict__ win,
               double *__restrict__ rout, const double *__restrict__ zin1,
               const double *__restrict__ zin2, double *__restrict__ zoutA,
               double *__restrict__ zoutB, const double *__restrict__ Kx,
-              const double *__restrict__ Ky, KArgs a, Region R, Region Dd, int ty, int jlim,
-              int step0, int restart) {
-    using G = TbGeom<M>;
+              const double *__restrict__ Ky, const double *__restrict__ pin,
+              double *__restrict__ pout, double *__restrict__ uio, KArgs a, Region R,
+              Region Dd, int ty, int jlim, int step0, int restart) {
+    constexpr int NL = M + (PRE ? 1 : 0) + (POST ? 1 : 0);  // stencil levels
+    constexpr int T0 = PRE ? 2 : 1;                         // level of the first Chebyshev step
+    using G = TbGeom<NL>;
     constexpr int D = G::D;
-    static_assert(M <= 6, "the TMEM ring holds M+2 rows");
+    static_assert(NL <= 6, "the TMEM ring holds NL+2 rows");
+    static_assert(!PRE || (FIRST && !FUSE && KG), "PRE: first pass, g faces, no FUSE update");
+    static_assert(!POST || LAST, "POST: last pass");
     static_assert(kTbW <= 4 || kTbW % 4 == 0, "warp quarters");
     extern __shared__ double2 tb_smem[];
     const double(*coef)[kMaxS] = c_tb_coef[a.coef_slot];
@@ -334,7 +329,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             cudaGraphSetConditional(a.cond, 0u);
         return;
     }
-    double alpha = 0.0;
+    double alpha = 0.0, beta = 0.0;
     if (FUSE) {
         const double pw = S->red_pw;
         alpha = S->gam_old / pw;
@@ -346,6 +341,18 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             }
             return;
         }
+    }
+    if (PRE) {
+        const Cg1Coef cf = cg1_coef(S);  // stop test on r.r, limits, alpha, beta
+        if (cf.state != 0) {
+            if (grid_arrive2(&S->ticket) && threadIdx.x == 0) {
+                cg1_finish(S, cf);
+                if (LAST && a.set_cond && a.cond) cudaGraphSetConditional(a.cond, 0u);
+            }
+            return;
+        }
+        alpha = cf.alpha;
+        beta = cf.beta;
     }
     trace_begin(a);
     const double2 z0 = make_double2(0.0, 0.0);
@@ -369,44 +376,29 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     for (int d = 0; d < D; ++d) tm_st16(tm + 16u * d, z0, z0, z0, z0);  // zero ring
 
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const int strip = blockIdx.x * kTbW + warp;
     // strips tile the output region R (which may reach into the halo on sides with a
-    // neighbour block: extended bounds); first strip starts MR before it.
-    // Shared edges: a CTA's warps march adjacent strips, the CTA loses MR columns per side.
-    const int jA = (kTbShare ? (R.j0 & ~1) - G::MR
-                             : (R.j0 & (TEA_TB_GEOM == 2 ? ~3 : ~1)) - G::SH) +
-                   (kTbShare ? blockIdx.x * G::OWC + warp * kStrip
-                             : (blockIdx.x * kTbW + warp) * G::OW) + 2 * lane;
-    const bool west_nb = kTbShare && warp > 0, east_nb = kTbShare && warp < kTbW - 1;
-    const int c_lo = west_nb ? 0 : (kTbShare ? G::MR : G::SH);
-    const int c_hi = east_nb ? kStrip : (kTbShare ? kStrip - G::MR : G::SH + G::OW);
+    // neighbour block: extended bounds); the first starts SH before it
+    const int jA = (R.j0 & (TEA_TB_GEOM == 2 ? ~3 : ~1)) - G::SH + strip * G::OW + 2 * lane;
     const int kt0 = R.k0 + blockIdx.y * ty;
     const int kt1 = min(kt0 + ty, R.k1);
     const int pitch = a.pitch;
     const bool ld_ok = jA + 1 < jlim;  // inside the allocation
-    // output columns: this strip's [MR, 64-MR) intersected with the region
+    // output columns: this strip's [SH, SH + OW) intersected with the region
     const int cA = 2 * lane, cB = 2 * lane + 1;
-    const bool oA = cA >= c_lo && cA < c_hi && jA >= R.j0 && jA < R.j1;
-    const bool oB = cB >= c_lo && cB < c_hi && jA + 1 >= R.j0 && jA + 1 < R.j1;
+    const bool oA = cA >= G::SH && cA < G::SH + G::OW && jA >= R.j0 && jA < R.j1;
+    const bool oB = cB >= G::SH && cB < G::SH + G::OW && jA + 1 >= R.j0 && jA + 1 < R.j1;
     // dot products over owned cells only (D), whatever the extension of R
     const bool dA = oA && jA >= Dd.j0 && jA < Dd.j1, dB = oB && jA + 1 >= Dd.j0 && jA + 1 < Dd.j1;
 
-    // stencil windows: W[t] holds z_t rows (oldest, middle, newest); W[0] = input operand
-    double2 W[M][3];
+    // stencil windows: W[t] holds level t's rows (oldest, middle, newest); W[0] = input
+    // operand (r, or p = z + beta p_old with PRE)
+    double2 W[NL][3];
 #pragma unroll
-    for (int t = 0; t < M; ++t) W[t][0] = W[t][1] = W[t][2] = z0;
-    // Shared strip edges, double-buffered by row parity: per warp and level t' < M the
-    // value row it produced this row-iteration -- lane 31's .y (the east warp's lane 0 west
-    // neighbour) and lane 0's Kx.x * value.x (the west warp's lane 31 east term) -- and
-    // lane 0's input-row Kx.x (the east face of the west warp's lane 31 cell B in diag(A)).
-    constexpr int NP = 2 * M + 1;
-    __shared__ double pub[2][kTbW][NP];
-    if (kTbShare) {
-        for (int i = threadIdx.x; i < 2 * kTbW * NP; i += kTbT) (&pub[0][0][0])[i] = 0.0;
-        __syncthreads();
-    }
-    double dot0 = 0.0, dot1 = 0.0;
+    for (int t = 0; t < NL; ++t) W[t][0] = W[t][1] = W[t][2] = z0;
+    double dot0 = 0.0, dot1 = 0.0, dot2 = 0.0;  // r.z, r.r (LAST); z.(A z) (POST)
 
-    const int kbeg = kt0 - M, kend = kt1 + M;
+    const int kbeg = kt0 - NL, kend = kt1 + NL;
     long long orow = (long long)kbeg * pitch + jA;  // offset of (jA, k); running, no k*pitch
     // Input rows are staged P rows ahead by cp.async into per-thread shared-memory slots
     // (each thread copies and later reads back only its own 16 B per stream, so no
@@ -420,7 +412,12 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         for (int q = 0; q < kTbNS; ++q) cpa[sl][q][threadIdx.x] = z0;
     auto issue = [&](long long o, int sl) {
         if (ld_ok) {
-            if (FIRST) {
+            if (PRE) {  // z_s, p_old, r, g, u
+                cp16(&cpa[sl][0][threadIdx.x], zin1 + o);
+                cp16(&cpa[sl][1][threadIdx.x], pin + o);
+                cp16(&cpa[sl][2][threadIdx.x], rin + o);
+                cp16(&cpa[sl][4][threadIdx.x], uio + o);
+            } else if (FIRST) {
                 cp16(&cpa[sl][0][threadIdx.x], rin + o);
                 if (FUSE) cp16(&cpa[sl][1][threadIdx.x], win + o);
             } else {
@@ -430,9 +427,6 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             }
             cp16(&cpa[sl][3][threadIdx.x], Kx + o);
             if (!KG) cp16(&cpa[sl][4][threadIdx.x], Ky + o);
-            // shared edges: lane 0 needs g(jA-1) for its west face (the west lane is in
-            // another warp) -- the 16-B pair g(jA-2), g(jA-1) into the free Ky slot
-            if (KG && kTbShare && lane == 0) cp16(&cpa[sl][4][threadIdx.x], Kx + o - 2);
         }
         cp_commit();  // one group per row, empty or not, so wait_group counts rows
     };
@@ -457,8 +451,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         double2 KX, KY;
         if (KG) {
             const double2 g = cpa[cs][3][threadIdx.x];
-            double gW = __shfl_up_sync(0xffffffffu, g.y, 1);
-            if (kTbShare && lane == 0) gW = cpa[cs][4][threadIdx.x].y;
+            const double gW = __shfl_up_sync(0xffffffffu, g.y, 1);
             // __dmul_rn: never contracted into an FMA with the faces' uses (the diagonal
             // sum below), so every face equals the stored one bit for bit
             KX.x = __dmul_rn(hrx, gW + g.x);
@@ -470,8 +463,12 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             KX = cpa[cs][3][threadIdx.x];
             KY = cpa[cs][4][threadIdx.x];
         }
-        double2 Wv = z0, Z2 = z0, RR = z0;
-        if (FIRST) {
+        double2 Wv = z0, Z2 = z0, RR = z0, PO = z0, UU = z0;
+        if (PRE) {
+            PO = cpa[cs][1][threadIdx.x];
+            RR = cpa[cs][2][threadIdx.x];
+            UU = cpa[cs][4][threadIdx.x];
+        } else if (FIRST) {
             if (FUSE) Wv = cpa[cs][1][threadIdx.x];
         } else {
             Z2 = cpa[cs][1][threadIdx.x];
@@ -487,129 +484,109 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             cs = cs == P ? 0 : cs + 1;
         }
         double2 rk;
-        if (FIRST) {
+        if (PRE) {
+            // level 0: p = z + beta p_old; u += alpha p (pointwise, this row)
+            X = make_double2(X.x + beta * PO.x, X.y + beta * PO.y);
+            if (k >= kt0 && k < kt1) {
+                st2m(pout + orow, X, oA, oB);
+                st2m(uio + orow, make_double2(UU.x + alpha * X.x, UU.y + alpha * X.y), oA, oB);
+            }
+            rk = RR;  // r_old: the w level replaces it by r - alpha A p
+        } else if (FIRST) {
             if (FUSE) X = make_double2(X.x - alpha * Wv.x, X.y - alpha * Wv.y);
             rk = X;
             if (FUSE && k >= kt0 && k < kt1) st2m(rout + orow, X, oA, oB);
         } else {
             rk = RR;
         }
-        // step t works on row q = k - t and needs that row's Kx, Ky, r (and Ky of row q+1):
-        // they wait in this thread's TMEM ring. The previous row's store must land before
-        // this row's loads read it back.
+        // level t works on row q = k - t and needs that row's Kx, Ky, r (and Ky of row
+        // q+1): they wait in this thread's TMEM ring. The previous row's stores must land
+        // before this row's loads read them back.
         tm_wait_st();
         tm_st12(tm + 16u * head, KX, KY, rk);
         TmRow tmA;
-        tm_ld12(tm + 16u * ((head - 1) & (D - 1)), tmA);  // row k-1: step 1's operands
+        tm_ld12(tm + 16u * ((head - 1) & (D - 1)), tmA);  // row k-1: level 1's operands
         tm_wait_ld(tmA);
         double2 s_kx = tm_get(tmA, 0), s_ky = tm_get(tmA, 1), s_r = tm_get(tmA, 2), kyn = KY;
-#if TEA_TB_DIAG
         // Row k-1 is completed now that its top faces (row k's Ky) are known: the diagonal
         // of A (Listing 1: 1 + the sum of the cell's four face coefficients) is formed once
-        // per row here, not once per step, and joins the row's slot (columns 12-15).
+        // per row here, not once per level, and joins the row's slot (columns 12-15).
         // Kx(jA+2) (the face east of cell B) is the east lane's Kx(jA): one shuffle per row
         // (lane 31's value only feeds the margin).
-        double kxE = __shfl_down_sync(0xffffffffu, s_kx.x, 1);
-        const int pb = (k - 1) & 1, cb = k & 1;  // parity buffers: previous row's, this row's
-        if (east_nb && lane == 31) kxE = pub[pb][warp + 1][2 * M];  // east warp's Kx(jA+2)
+        const double kxE = __shfl_down_sync(0xffffffffu, s_kx.x, 1);
         double2 s_d;
         s_d.x = 1.0 + (s_kx.x + s_kx.y) + (s_ky.x + KY.x);
         s_d.y = 1.0 + (s_kx.y + kxE) + (s_ky.y + KY.y);
         tm_st4(tm + 16u * ((head - 1) & (D - 1)) + 12u, s_d);
-#endif
         const double2 z2row = z2prev;  // z_{i-2} of row k-1
         if (!FIRST) z2prev = Z2;
         W[0][0] = W[0][1];
         W[0][1] = W[0][2];
         W[0][2] = X;
-        if (kTbShare) {
-            if (lane == 0) {
-                pub[cb][warp][0] = KX.x * X.x;
-                pub[cb][warp][2 * M] = KX.x;
-            }
-            if (lane == 31) pub[cb][warp][1] = X.y;
-        }
 #pragma unroll
-        for (int t = 1; t <= M; ++t) {
+        for (int t = 1; t <= NL; ++t) {
             const int q = k - t;
-            // issue the next step's slot (row q-1) before computing this one
+            // issue the next level's slot (row q-1) before computing this one
             TmRow tmB;
-#if TEA_TB_DIAG
-            if (t < M) tm_ld16(tm + 16u * ((head - t - 1) & (D - 1)), tmB);
-#else
-            if (t < M) tm_ld12(tm + 16u * ((head - t - 1) & (D - 1)), tmB);
-#endif
+            if (t < NL) tm_ld16(tm + 16u * ((head - t - 1) & (D - 1)), tmB);
             const double2 kx = s_kx, kyc = s_ky, rq = s_r;
-            double2 z2;
-            if (t == 1) {
-                z2 = FIRST ? z0 : z2row;
-            } else {
-                z2 = W[t >= 2 ? t - 2 : 0][0];
-            }
             const double2 xm = W[t - 1][0], xc = W[t - 1][1], xp = W[t - 1][2];
-            const int ci = step0 - 2 + t;
-            const double cx = coef[0][ci], cz = coef[1][ci], cr = coef[2][ci], ca = coef[3][ci];
+            const double2 dg = s_d;
             // lane 0's left and lane 31's right neighbours are outside the strip: the
             // shuffles return the lane's own (finite) value, which only pollutes the
-            // overlap columns every step already discards -- no selects needed.
-            // Dependency order: xp (the "up" row) is the row step t-1 produced in THIS
-            // row-iteration; everything else is older. Form the rest first, fold xp in last.
-            double2 zn;
-#if TEA_TB_DIAG
-            // z = cx X + cz z2 + cr r - ca (d X - sum_f K_f X_f)              (Listing 1)
+            // overlap columns every level already discards -- no selects needed.
             // West neighbour of cell A from the west lane; the east term of cell B,
             // Kx(jA+2) X(jA+2), is the east lane's own Kx(jA) X(jA) -- one product shuffled.
-            // The per-step coefficients only ever multiply vector registers (uniform
-            // operands, nothing hoisted into vector registers).
-            const double2 dg = s_d;
-            double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
-            double east = __shfl_down_sync(0xffffffffu, kx.x * xc.x, 1);
-            if (west_nb && lane == 0) left = pub[pb][warp - 1][2 * (t - 1) + 1];
-            if (east_nb && lane == 31) east = pub[pb][warp + 1][2 * (t - 1)];
-            double2 base, nb;
-            base.x = cx * xc.x;
-            base.y = cx * xc.y;
-            if (!(FIRST && t == 1)) {
-                base.x = fma(cz, z2.x, base.x);
-                base.y = fma(cz, z2.y, base.y);
-            }
-            base.x = fma(cr, rq.x, base.x);
-            base.y = fma(cr, rq.y, base.y);
+            // Dependency order: xp (the "up" row) is the row level t-1 produced in THIS
+            // row-iteration; everything else is older. Form the rest first, fold xp in last.
+            const double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
+            const double east = __shfl_down_sync(0xffffffffu, kx.x * xc.x, 1);
+            double2 nb;  // sum_f K_f X_f - d X without the up face (Listing 1)
             nb.x = fma(-dg.x, xc.x, fma(kx.x, left, fma(kx.y, xc.y, kyc.x * xm.x)));
             nb.y = fma(-dg.y, xc.y, fma(kx.y, xc.x, fma(kyc.y, xm.y, east)));
-            // (folding ca into kyn to leave one dependent DFMA after xp costs a DMUL per cell
-            // and measured slower: profiles/r01g_tmem_cpa.txt)
-            zn.x = fma(ca, fma(kyn.x, xp.x, nb.x), base.x);
-            zn.y = fma(ca, fma(kyn.y, xp.y, nb.y), base.y);
-#else
-            // x direction in flux form: A x = x + sum_faces K_f (x_c - x_f) (Listing 1
-            // regrouped). gw = Kx_w (x_A - x_left) is formed by the lane that owns the face's
-            // Kx; its east neighbour receives it as -(its east flux).
-            const double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
-            const double gw = kx.x * (xc.x - left);
-            const double gm = kx.y * (xc.x - xc.y);
-            const double ge = __shfl_down_sync(0xffffffffu, gw, 1);  // Kx_e (x_right - x_B)
-            double2 AXo, base;  // A x without the up term; the step's x-independent part
-            AXo.x = (1.0 + (kyn.x + kyc.x)) * xc.x - kyc.x * xm.x + (gw + gm);
-            AXo.y = (1.0 + (kyn.y + kyc.y)) * xc.y - kyc.y * xm.y - (gm + ge);
-            base.x = cx * xc.x + cz * z2.x + cr * rq.x;
-            base.y = cx * xc.y + cz * z2.y + cr * rq.y;
-            zn.x = fma(-ca, fma(-kyn.x, xp.x, AXo.x), base.x);
-            zn.y = fma(-ca, fma(-kyn.y, xp.y, AXo.y), base.y);
-#endif
             const bool rowout = q >= kt0 && q < kt1;
-            if (t < M) {
-                const int tt = t < M ? t : M - 1;
-                W[tt][0] = W[tt][1];
-                W[tt][1] = W[tt][2];
-                W[tt][2] = zn;
-                if (kTbShare) {
-                    if (lane == 0) pub[cb][warp][2 * tt] = kx.x * zn.x;
-                    if (lane == 31) pub[cb][warp][2 * tt + 1] = zn.y;
+            double2 zn = z0;
+            if (PRE && t == 1) {
+                // w = A p; r' = r - alpha w = r + alpha (sum_f K_f p_f - d p)
+                zn.x = fma(alpha, fma(kyn.x, xp.x, nb.x), rq.x);
+                zn.y = fma(alpha, fma(kyn.y, xp.y, nb.y), rq.y);
+                tm_st4(tm + 16u * ((head - 1) & (D - 1)) + 8u, zn);  // row q's r is now r'
+                if (rowout) st2m(rout + (orow - pitch), zn, oA, oB);
+            } else if (POST && t == NL) {
+                // q = A z_s at row q (xc = z_s): z_s . q over the owned cells
+                if (rowout && q >= Dd.k0 && q < Dd.k1) {
+                    const double mx = fma(kyn.x, xp.x, nb.x), my = fma(kyn.y, xp.y, nb.y);
+                    if (dA) dot2 -= xc.x * mx;
+                    if (dB) dot2 -= xc.y * my;
                 }
-                if (t == M - 1 && !LAST && rowout) st2m(zoutA + (orow - t * pitch), zn, oA, oB);
             } else {
-                if (rowout) {
+                // Chebyshev step j of this pass (DESIGN.md §4.3 recurrence):
+                // z = cx X + cz z2 + cr r - ca (d X - sum_f K_f X_f)         (Listing 1)
+                // The per-step coefficients only ever multiply vector registers (uniform
+                // operands, nothing hoisted into vector registers).
+                const int j = t - (PRE ? 1 : 0);
+                const int ci = step0 - 2 + j;
+                const double cx = coef[0][ci], cz = coef[1][ci], cr = coef[2][ci], ca = coef[3][ci];
+                double2 z2 = z0;
+                if (t == 1)
+                    z2 = FIRST ? z0 : z2row;
+                else if (!(FIRST && t == T0))
+                    z2 = W[t >= 2 ? t - 2 : 0][0];
+                double2 base;
+                base.x = cx * xc.x;
+                base.y = cx * xc.y;
+                if (!(FIRST && t == T0)) {
+                    base.x = fma(cz, z2.x, base.x);
+                    base.y = fma(cz, z2.y, base.y);
+                }
+                base.x = fma(cr, rq.x, base.x);
+                base.y = fma(cr, rq.y, base.y);
+                // (folding ca into kyn to leave one dependent DFMA after xp costs a DMUL per
+                // cell and measured slower: profiles/r01g_tmem_cpa.txt)
+                zn.x = fma(ca, fma(kyn.x, xp.x, nb.x), base.x);
+                zn.y = fma(ca, fma(kyn.y, xp.y, nb.y), base.y);
+                if (j == M - 1 && !LAST && rowout) st2m(zoutA + (orow - t * pitch), zn, oA, oB);
+                if (j == M && rowout) {
                     st2m(zoutB + (orow - t * pitch), zn, oA, oB);
                     if (LAST && q >= Dd.k0 && q < Dd.k1) {
                         if (dA) {
@@ -623,18 +600,19 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                     }
                 }
             }
-            if (t < M) {
+            if (t < NL) {
+                const int tt = t < NL ? t : NL - 1;
+                W[tt][0] = W[tt][1];
+                W[tt][1] = W[tt][2];
+                W[tt][2] = zn;
                 tm_wait_ld(tmB);
                 kyn = kyc;  // Ky of row q = the top faces of row q-1
                 s_kx = tm_get(tmB, 0);
                 s_ky = tm_get(tmB, 1);
                 s_r = tm_get(tmB, 2);
-#if TEA_TB_DIAG
                 s_d = tm_get(tmB, 3);
-#endif
             }
         }
-        if (kTbShare) __syncthreads();  // this row's edges published before the next row
     }
     asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory");
     __syncthreads();
@@ -643,17 +621,41 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                      "n"(kTmAlloc)
                      : "memory");
     if (LAST) {
-        double t0, t1;
-        if (grid_reduce2(dot0, dot1, a.partials, &S->ticket, &t0, &t1)) {
-            if (threadIdx.x == 0) {
-                S->red_gam = t0;
-                S->red_rr = t1;
-                if (FUSE) S->alpha_prev = alpha;
-                if (!restart) {
-                    S->it += 1;
-                    S->outer += 1;
-                }
+        bool last;
+        double tot[3] = {0.0, 0.0, 0.0};
+        if (POST) {
+            const double v[3] = {dot0, dot1, dot2};
+            last = grid_reduce_n<3>(v, a.partials, &S->ticket, tot);
+        } else {
+            const double v[2] = {dot0, dot1};
+            double t2[2];
+            last = grid_reduce_n<2>(v, a.partials, &S->ticket, t2);
+            tot[0] = t2[0];
+            tot[1] = t2[1];
+        }
+        if (last && threadIdx.x == 0) {
+            if (PRE) {  // this iteration's alpha, beta (before the new gamma replaces it)
+                S->gam_old = S->red_gam;
+                S->alpha_prev = alpha;
+                S->beta_last = beta;
+                S->fresh = 0;
             }
+            S->red_gam = tot[0];
+            S->red_rr = tot[1];
+            if (POST) S->red_pw = tot[2];
+            if (FUSE) S->alpha_prev = alpha;
+            if (!restart) {
+                S->it += 1;
+                S->outer += 1;
+            }
+        }
+    } else if (PRE) {
+        // every CTA has read the scalars (it arrived): the last one records this iteration's
+        if (grid_arrive2(&S->ticket) && threadIdx.x == 0) {
+            S->gam_old = S->red_gam;
+            S->alpha_prev = alpha;
+            S->beta_last = beta;
+            S->fresh = 0;
         }
     } else if (FUSE) {
         if (blockIdx.x == 0 && blockIdx.y == 0 && blockIdx.z == 0 && threadIdx.x == 0) S->alpha_prev = alpha;
@@ -661,50 +663,68 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     trace_end(a);
 }
 
-// output columns of one CTA of an M-step pass
-int tb_out_cols(int M) {
-    const int mr = (M + 1) & ~1;
-    const int ow = TEA_TB_GEOM == 0 ? kStrip - 2 * M : (TEA_TB_GEOM == 2 ? 48 : kStrip - 2 * mr);
-    return kTbShare ? kTbW * kStrip - 2 * mr : kTbW * ow;
+// output columns of one CTA of a pass with NL stencil levels
+int tb_out_cols(int NL) {
+    const int mr = (NL + 1) & ~1;
+    const int ow = TEA_TB_GEOM == 0 ? kStrip - 2 * NL : (TEA_TB_GEOM == 2 ? 48 : kStrip - 2 * mr);
+    return kTbW * ow;
 }
 
-template <int M, bool FIRST, bool FUSE, bool LAST, bool KG>
+template <int M, bool FIRST, bool FUSE, bool LAST, bool KG, bool PRE, bool POST>
 static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty, int jlim,
-                      int step0, bool restart,
-                      const double *rin, const double *win, double *rout, const double *zin1,
-                      const double *zin2, double *zoutA, double *zoutB, const double *kx,
-                      const double *ky, cudaStream_t st) {
-    using G = TbGeom<M>;
-    const int width = R.j1 - (R.j0 & ~1);
-    dim3 grid((width + G::OWC - 1) / G::OWC, (R.k1 - R.k0 + ty - 1) / ty);
+                      int step0, bool restart, const TbArgs &f, cudaStream_t st) {
+    constexpr int NL = M + (PRE ? 1 : 0) + (POST ? 1 : 0);
+    const int width = R.j1 - (R.j0 & (TEA_TB_GEOM == 2 ? ~3 : ~1));
+    const int ow = tb_out_cols(NL);
+    dim3 grid((width + ow - 1) / ow, (R.k1 - R.k0 + ty - 1) / ty);
     constexpr size_t smem = tb_smem_bytes();
     // > 48 KB of dynamic shared memory needs the attribute, set once per device
     static std::atomic<unsigned long long> attr{0ull};  // per instantiation: device bit mask
     const unsigned long long bit = 1ull << tea_device();
     if (!(attr.load() & bit)) {
-        cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST, KG>,
+        cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST, KG, PRE, POST>,
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         attr.fetch_or(bit);
     }
-    k_cheb_tb<M, FIRST, FUSE, LAST, KG><<<grid, kTbT, smem, st>>>(
-        rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, a, R, Dd, ty, jlim, step0, restart ? 1 : 0);
+    k_cheb_tb<M, FIRST, FUSE, LAST, KG, PRE, POST><<<grid, kTbT, smem, st>>>(
+        f.rin, f.win, f.rout, f.zin1, f.zin2, f.zoutA, f.zoutB, KG ? a.g : f.kx, f.ky, f.pin,
+        f.pout, f.uio, a, R, Dd, ty, jlim, step0, restart ? 1 : 0);
 }
 
 template <int M>
 static void tb_dispatch(const KArgs &a, const Region &R, const Region &Dd, int ty, int jlim,
-                        int step0, bool first,
-                        bool fuse, bool last, bool restart, const double *rin, const double *win,
-                        double *rout, const double *zin1, const double *zin2, double *zoutA,
-                        double *zoutB, const double *kx, const double *ky, cudaStream_t st) {
-#define TB(F, U, L)                                                                            \
-    do {                                                                                       \
-        if (a.g)                                                                               \
-            tb_launch<M, F, U, L, true>(a, R, Dd, ty, jlim, step0, restart, rin, win, rout, zin1, \
-                                        zin2, zoutA, zoutB, a.g, nullptr, st);                 \
-        else                                                                                   \
-            tb_launch<M, F, U, L, false>(a, R, Dd, ty, jlim, step0, restart, rin, win, rout,     \
-                                         zin1, zin2, zoutA, zoutB, kx, ky, st);                \
+                        int step0, bool first, bool fuse, bool last, bool restart, bool pre,
+                        bool post, const TbArgs &f, cudaStream_t st) {
+#define TB(F, U, L)                                                                       \
+    do {                                                                                  \
+        if (a.g)                                                                          \
+            tb_launch<M, F, U, L, true, false, false>(a, R, Dd, ty, jlim, step0, restart, f, st); \
+        else                                                                              \
+            tb_launch<M, F, U, L, false, false, false>(a, R, Dd, ty, jlim, step0, restart, f, st); \
     } while (0)
+    if (pre || post) {
+        // single-reduction CPPCG in fused form (faces from g only; at most 6 levels)
+        if constexpr (M <= 4) {
+            if (pre && post) {
+                tb_launch<M, true, false, true, true, true, true>(a, R, Dd, ty, jlim, step0, restart, f, st);
+                return;
+            }
+        }
+        if constexpr (M <= 5) {
+            if (pre && !post && first && !last) {
+                tb_launch<M, true, false, false, true, true, false>(a, R, Dd, ty, jlim, step0, restart, f, st);
+                return;
+            }
+            if (post && !pre && last) {
+                if (first)
+                    tb_launch<M, true, false, true, true, false, true>(a, R, Dd, ty, jlim, step0, restart, f, st);
+                else
+                    tb_launch<M, false, false, true, true, false, true>(a, R, Dd, ty, jlim, step0, restart, f, st);
+                return;
+            }
+        }
+        return;  // invalid combination (the host plans only the ones above)
+    }
     if (first) {
         if (fuse) {
             if (last) TB(true, true, true); else TB(true, true, false);
@@ -719,72 +739,66 @@ static void tb_dispatch(const KArgs &a, const Region &R, const Region &Dd, int t
 
 int tb_max_steps() { return 5; }
 
-// Rows per CTA tile: a CTA costs ~ (ty + 2M) row-iterations (pipeline fill/drain), all
-// CTAs are alike, so a launch costs ~ waves x (ty + 2M) with waves = ceil(ctas / slots).
-// Pick ty minimising that (slots = SMs x resident CTAs per SM of this kernel).
-int tb_auto_rows(int M, int width, int height) {
+// Rows per CTA tile: a CTA costs ~ (ty + 2 NL) row-iterations (pipeline fill/drain), all
+// CTAs are alike, so a launch costs ~ waves x (ty + 2 NL) with waves = ceil(ctas / slots).
+// Pick ty minimising that (slots = SMs x resident CTAs per SM of a pass with NL levels).
+int tb_auto_rows(int NL, int width, int height) {
     static std::atomic<int> slot_cache[kMaxDev][8];
-    M = M < 1 ? 1 : (M > kTbMaxSteps ? kTbMaxSteps : M);
+    NL = NL < 1 ? 1 : (NL > 6 ? 6 : NL);
     const int dev = tea_device();
-    int slots_m = slot_cache[dev][M].load();
-    if (!slots_m) {
+    int slots = slot_cache[dev][NL].load();
+    if (!slots) {
         int nsm = 148, per = 0;
         cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, dev);
         const size_t smem = tb_smem_bytes();
         cudaError_t e = cudaSuccess;
-        switch (M) {
-#define OCC(m)                                                                                   \
-    case m:                                                                                      \
-        cudaFuncSetAttribute(k_cheb_tb<m, false, false, true, true>,                             \
+        switch (NL) {
+#define OCC(m, POST)                                                                             \
+    case (m + (POST ? 1 : 0)):                                                                   \
+        cudaFuncSetAttribute(k_cheb_tb<m, false, false, true, true, false, POST>,                \
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);            \
-        e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per,                                  \
-                                                          k_cheb_tb<m, false, false, true, true>, \
-                                                          kTbT, smem);                       \
+        e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(                                       \
+            &per, k_cheb_tb<m, false, false, true, true, false, POST>, kTbT, smem);              \
         break;
-            OCC(1) OCC(2) OCC(3) OCC(4) OCC(5)
+            OCC(1, false) OCC(2, false) OCC(3, false) OCC(4, false) OCC(5, false) OCC(5, true)
 #undef OCC
         }
         if (e != cudaSuccess || per < 1) per = 1;
-        slots_m = nsm * per;
-        slot_cache[dev][M].store(slots_m);
+        slots = nsm * per;
+        slot_cache[dev][NL].store(slots);
     }
-    int slots[8] = {};
-    slots[M] = slots_m;
-    const int ow = tb_out_cols(M);
+    const int ow = tb_out_cols(NL);
     const int gx = (width + ow - 1) / ow;
     int best = height, bestc = 0x7fffffff;
     for (int w = 1; w <= 256; ++w) {
-        const int tiles = (int)((long long)slots[M] * w / gx);
+        const int tiles = (int)((long long)slots * w / gx);
         if (tiles < 1) continue;
         const int ty = (height + tiles - 1) / tiles;
-        const int waves = (int)(((long long)gx * ((height + ty - 1) / ty) + slots[M] - 1) / slots[M]);
-        const long long cost = (long long)waves * (ty + 2 * M);
+        const int waves = (int)(((long long)gx * ((height + ty - 1) / ty) + slots - 1) / slots);
+        const long long cost = (long long)waves * (ty + 2 * NL);
         if (cost < bestc) {
             bestc = (int)cost;
             best = ty;
         }
-        if (ty <= 2 * M) break;
+        if (ty <= 2 * NL) break;
     }
     return best < 1 ? 1 : best;
 }
 
-int tb_ctas(int M, int width, int height, int ty) {
-    const int ow = tb_out_cols(M);
+int tb_ctas(int NL, int width, int height, int ty) {
+    const int ow = tb_out_cols(NL);
     return ((width + ow - 1) / ow) * ((height + ty - 1) / ty);
 }
 
 void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, int ty, int jlim,
-                    int step0,
-                    bool first, bool fuse, bool last, bool restart, const double *rin,
-                    const double *win, double *rout, const double *zin1, const double *zin2,
-                    double *zoutA, double *zoutB, const double *kx, const double *ky,
-                    cudaStream_t st) {
+                    int step0, bool first, bool fuse, bool last, bool restart, bool pre,
+                    bool post, const TbArgs &f, cudaStream_t st) {
     switch (M) {
-        case 1: tb_dispatch<1>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
-        case 2: tb_dispatch<2>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
-        case 3: tb_dispatch<3>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
-        case 4: tb_dispatch<4>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
-        default: tb_dispatch<5>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, rin, win, rout, zin1, zin2, zoutA, zoutB, kx, ky, st); break;
+        case 1: tb_dispatch<1>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, f, st); break;
+        case 2: tb_dispatch<2>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, f, st); break;
+        case 3: tb_dispatch<3>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, f, st); break;
+        case 4: tb_dispatch<4>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, f, st); break;
+        default: tb_dispatch<5>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, f, st); break;
     }
 }
 

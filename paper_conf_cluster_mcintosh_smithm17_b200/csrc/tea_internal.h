@@ -72,6 +72,39 @@ struct Region {
     int j0, j1, k0, k1;
 };
 
+// Chronopoulos & Gear scalars of the single-reduction methods (CG1, CPPCG1, CPPCG1F), from the
+// last reduction: red_gam = gamma_i, red_pw = delta_i, red_rr = r.r; gam_old = gamma_{i-1},
+// alpha_prev = alpha_{i-1}; fresh marks i = 0 (beta = 0, alpha = gamma/delta).
+struct Cg1Coef {
+    double alpha, beta;
+    int state;  // 0 run, 1 converged, 2 limit, 3 breakdown
+};
+__device__ __forceinline__ Cg1Coef cg1_coef(const Scalars *S) {
+    Cg1Coef c{0.0, 0.0, 0};
+    const double gam = S->red_gam, del = S->red_pw;
+    // stop test on ||r|| (reading R5): red_rr = r.r (= gam for CG1, where z = r)
+    if (!S->fresh && sqrt(S->red_rr) < S->eps * S->r0) {
+        c.state = 1;
+        return c;
+    }
+    if (S->it >= S->it_limit) {
+        c.state = 2;
+        return c;
+    }
+    double den = del;
+    if (!S->fresh) {
+        c.beta = gam / S->gam_old;
+        den = del - c.beta * gam / S->alpha_prev;
+    }
+    c.alpha = gam / den;
+    if (!(den > 0.0) || !isfinite(c.alpha)) c.state = 3;
+    return c;
+}
+__device__ __forceinline__ void cg1_finish(Scalars *S, const Cg1Coef &c) {
+    S->done = 1;
+    S->status = c.state == 1 ? DS_CONVERGED : (c.state == 2 ? DS_LIMIT : DS_BREAKDOWN);
+}
+
 // Field indices inside a block's workspace.
 enum Field {
     F_U0 = 0, F_U, F_KX, F_KY, F_KZ, F_R0, F_R1, F_P0, F_P1, F_W, F_Z0, F_Z1, F_Z2, F_Z3,
@@ -217,19 +250,34 @@ void launch_cg1_update(const KArgs &a, const Launch &L, const Region &R, const d
 void launch_cg1_w(const KArgs &a, const Launch &L, const Region &R, const double *r, double *w,
                   const double *kx, const double *ky, cudaStream_t st, bool pw_only = false);
 
+// Single-reduction CPPCG, fused form (CPPCG1F): the outer update as one stencil pass
+// (p = z + b p on R + ring, w = A p, r -= a w, u += a p), where the fused passes do not.
+void launch_cg1f_pre(const KArgs &a, const Launch &L, const Region &R, const double *z,
+                     const double *pin, double *pout, double *r, double *u, const double *kx,
+                     const double *ky, cudaStream_t st);
+
 // Temporally blocked Chebyshev passes (tea_cheb_tb.cu).
 constexpr int kTbMaxSteps = 5;
-int tb_out_cols(int M);
-int tb_ctas(int M, int width, int height, int ty);
-int tb_auto_rows(int M, int width, int height);
+struct TbArgs {
+    const double *rin = nullptr, *win = nullptr;    // r (in), w (FUSE update)
+    double *rout = nullptr;                         // r' (FUSE / PRE)
+    const double *zin1 = nullptr, *zin2 = nullptr;  // z_{i-1}, z_{i-2} (later passes; PRE: z_s)
+    double *zoutA = nullptr, *zoutB = nullptr;      // z_{last-1}, z_last
+    const double *kx = nullptr, *ky = nullptr;      // stored faces (kform -1)
+    const double *pin = nullptr;                    // PRE: p_old
+    double *pout = nullptr, *uio = nullptr;         // PRE: p, u (in place)
+};
+int tb_out_cols(int levels);
+int tb_ctas(int levels, int width, int height, int ty);
+int tb_auto_rows(int levels, int width, int height);
 int tb_slot_acquire();  // -1: none free (the context then uses per-step kernels)
 void tb_slot_release(int slot);
 cudaError_t tb_coef_upload(int slot, const Scalars *S, cudaStream_t st);
+// M Chebyshev steps in one pass; pre: the CPPCG1F outer update first (first pass, g faces),
+// post: q = A z_s and z_s.q after the last step (last pass, g faces)
 void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, int ty, int jlim,
-                    int step0, bool first, bool fuse, bool last, bool restart, const double *rin,
-                    const double *win, double *rout, const double *zin1, const double *zin2,
-                    double *zoutA, double *zoutB, const double *kx, const double *ky,
-                    cudaStream_t st);
+                    int step0, bool first, bool fuse, bool last, bool restart, bool pre,
+                    bool post, const TbArgs &f, cudaStream_t st);
 
 // Persistent single-launch CG / CPPCG solve of one 2D block (tea_kernels.cu, k_persist):
 // phases separated by grid-wide barriers of a cooperative launch.

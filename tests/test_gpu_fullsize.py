@@ -58,14 +58,14 @@ def oracle_case(ora, n, method, its):
     return _cache[key]
 
 
-@pytest.mark.parametrize("method,its", [(0, 50), (1, 33)])
+@pytest.mark.parametrize("method,its", [(0, 50), (1, 33), (7, 33)])
 @pytest.mark.parametrize("blocks", [None, (2, 4)])
 def test_4096_every_cell(tea, ora, method, its, blocks):
     deck, u_o, st_o, s_o = oracle_case(ora, 4096, method, its)
     dist = None
     if blocks:
         dist = dict(rank=0, nranks=1, px=blocks[0], py=blocks[1],
-                    halo_depth=11 if method == 1 else 1)
+                    halo_depth=11 if method in (1, 7) else 1)
     u_g, r = gpu_run(tea, deck, dist, method=method, eps=0.0, max_iters=its, inner_steps=10)
     err = pointwise(u_g, u_o)
     print(f"\n4096^2 method={method} its={its} blocks={blocks}: max pointwise rel err "
@@ -74,7 +74,7 @@ def test_4096_every_cell(tea, ora, method, its, blocks):
     assert s_o == 1 and r.status == 1  # TEA_NOT_CONVERGED: the fixed count was run
     assert r.stats["iterations"] == st_o["iterations"] == its
     assert r.stats["rnorm"] == pytest.approx(st_o["rnorm"], rel=1e-9)
-    if method == 1:
+    if method in (1, 7):
         assert r.stats["presteps"] == st_o["presteps"] == 30
         assert r.stats["outer"] == st_o["outer"] == its - 30
         assert r.stats["eig_min"] == pytest.approx(st_o["eig_min"], rel=1e-9)

@@ -743,3 +743,78 @@ def test_kform_bitwise_blocks(tea, ora, blocks, d, method):
     u_o, st_o, _ = ora.run(deck, steps=1, **kw)
     assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
     assert field_err(u_g, u_o, "random") <= 1e-10
+
+
+# ---------------------------------------------------------------- single-reduction CPPCG, fused
+# TEA_CPPCG1F (oracle ORA_CPPCG1F, reading R23): one block with the fused passes = two kernels
+# per outer iteration (the first pass carries the outer update, the last q = A z_s and the
+# three dots); blocks / one kernel per step: k_cg1f_pre + chain (+ k_cg1_w) + one reduction.
+@pytest.mark.parametrize("kind,nx,ny,s,tb", [("pipe", 128, 128, 10, 0), ("pipe", 256, 200, 10, 5),
+                                             ("pipe", 256, 200, 10, 1), ("random", 300, 203, 4, 0),
+                                             ("random", 97, 61, 3, 5), ("random", 1000, 777, 10, 0),
+                                             ("random", 257, 65, 7, 4), ("random", 1, 97, 6, 5),
+                                             ("random", 95, 1, 6, 5)])
+def test_cppcg1f_converged(tea, ora, kind, nx, ny, s, tb):
+    deck = deck_of(kind, nx, ny, seed=6)
+    kw = dict(method=7, eps=1e-13, max_iters=20000, inner_steps=s)
+    u_o, st_o, s_o = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, tb_steps=tb, persist=-1, **kw)
+    assert s_o[0] == 0 and st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    if st_g[0]["outer"] > 0 and st_o[0]["outer"] > 0:  # (1-wide decks can converge at the
+        assert st_g[0]["presteps"] == st_o[0]["presteps"]  # prestep boundary, +-1)
+        assert st_g[0]["matvecs"] == 1 + st_g[0]["presteps"] + s + 1 + st_g[0]["outer"] * (s + 2)
+    assert field_err(u_g, u_o, kind) <= 1e-10
+    u_c, st_c = gpu_run(tea, deck, tb_steps=tb, persist=-1, **dict(kw, method=1))
+    assert abs(st_c[0]["outer"] - st_g[0]["outer"]) <= 2
+    assert rel_err(u_g, u_c) <= 1e-10
+
+
+@pytest.mark.parametrize("s", [2, 3, 4, 5, 7, 10, 11, 13])
+def test_cppcg1f_pass_splits(tea, ora, s):
+    """Every inner-step count: the one-block fused path splits the chain into an even number
+    of passes (the first pass's output never aliases the z_s it reads), pre + post levels."""
+    deck = deck_of("pipe", 256, 200)
+    kw = dict(method=7, eps=1e-13, max_iters=20000, inner_steps=s)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, tb_steps=5, persist=-1, **kw)
+    assert st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+
+
+@pytest.mark.parametrize("k", [1, 2, 7])
+@pytest.mark.parametrize("tb", [1, 3, 5])
+def test_cppcg1f_fixed_iterations(tea, ora, k, tb):
+    deck = deck_of("random", 300, 203, seed=8, dt=0.04)
+    kw = dict(method=7, eps=0.0, max_iters=30 + k, inner_steps=10)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, tb_steps=tb, persist=-1, **kw)
+    assert st_g[0]["iterations"] == 30 + k and st_g[0]["outer"] == k
+    assert iter_err(u_g, u_o, "random") <= 1e-12
+    assert float(np.max(np.abs(u_g - u_o))) <= residual_bound(ora, deck, u_g, u_o)
+    assert st_g[0]["rnorm"] == pytest.approx(st_o[0]["rnorm"], rel=1e-9)
+
+
+@pytest.mark.parametrize("px,py,d,tb", [(2, 1, 11, 5), (2, 2, 11, 5), (3, 2, 12, 4), (1, 3, 2, 0),
+                                        (4, 2, 4, 0), (2, 2, 1, 0)])
+@pytest.mark.parametrize("loop_mode", [0, 2])
+def test_cppcg1f_multiblock(tea, ora, px, py, d, tb, loop_mode):
+    deck = deck_of("pipe", 200, 170)
+    kw = dict(method=7, eps=1e-13, max_iters=20000, inner_steps=10)
+    u_o, st_o, _ = ora.run(deck, steps=1, **kw)
+    u_g, st_g = gpu_run(tea, deck, dist=dict(px=px, py=py, halo_depth=d, nranks=1), tb_steps=tb,
+                        loop_mode=loop_mode, **kw)
+    assert st_g[0]["ret"] == 0
+    assert abs(st_g[0]["iterations"] - st_o[0]["iterations"]) <= 2
+    assert rel_err(u_g, u_o) <= 1e-10
+
+
+@pytest.mark.parametrize("loop_mode", [1, 2])
+def test_cppcg1f_loop_modes_identical(tea, loop_mode):
+    deck = deck_of("pipe", 1000, 700)
+    kw = dict(method=7, eps=1e-12, max_iters=5000, inner_steps=10)
+    ref, st_ref = gpu_run(tea, deck, **kw)
+    u, st = gpu_run(tea, deck, loop_mode=loop_mode, check_interval=6, **kw)
+    assert st[0]["iterations"] == st_ref[0]["iterations"]
+    assert np.array_equal(u, ref)
