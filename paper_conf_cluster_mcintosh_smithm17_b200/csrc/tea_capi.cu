@@ -767,6 +767,8 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
 // chain at once (d >= s + 1, the paper's deep-halo regime)
 bool use_tb(tea_ctx *c, int s) {
     if (is3d(c) || tb_steps(c) <= 1 || c->coef_slot < 0) return false;
+    // the passes address a field with 32-bit offsets
+    if ((double)c->blocks[0].L.rows * c->blocks[0].L.pitch >= 2147483648.0) return false;
     return single_block(c) || c->d >= s + 1;
 }
 // CPPCG1F: the pre / post levels form faces from g (kform >= 0) and need >= 2 passes

@@ -76,13 +76,30 @@ cudaError_t tb_coef_upload(int slot, const Scalars *S, cudaStream_t st) {
 
 namespace {
 
+#ifndef TEA_TB_PSTORE
+#define TEA_TB_PSTORE 1
+#endif
+// Store the lane's pair where a / b: predicated stores (one 16-B store, or one 8-B half at a
+// region edge) instead of branches -- no reconvergence blocks in the row loop.
 __device__ __forceinline__ void st2m(double *p, double2 v, bool a, bool b) {
+#if TEA_TB_PSTORE
+    const int ab = a && b, oa = a && !b, ob = b && !a;
+    asm volatile(
+        "{\n\t.reg .pred q0, q1, q2;\n\t"
+        "setp.ne.s32 q0, %3, 0;\n\tsetp.ne.s32 q1, %4, 0;\n\tsetp.ne.s32 q2, %5, 0;\n\t"
+        "@q0 st.global.v2.f64 [%0], {%1, %2};\n\t"
+        "@q1 st.global.f64 [%0], %1;\n\t"
+        "@q2 st.global.f64 [%0+8], %2;\n\t}" ::"l"(p),
+        "d"(v.x), "d"(v.y), "r"(ab), "r"(oa), "r"(ob)
+        : "memory");
+#else
     if (a && b) {
         *reinterpret_cast<double2 *>(p) = v;
     } else {
         if (a) p[0] = v.x;
         if (b) p[1] = v.y;
     }
+#endif
 }
 __device__ __forceinline__ void cp16(void *sdst, const double *gsrc) {
     asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(
@@ -263,6 +280,9 @@ constexpr size_t tb_smem_bytes() {
                : 48u * 1024u;
 }
 
+#ifndef TEA_TB_RING6
+#define TEA_TB_RING6 1
+#endif
 // Strip geometry: a warp's 64 columns output [SH, SH + OW); strips start SH before the
 // region at a stride of OW. 1 (default): SH = MR = levels rounded up to even, OW = 64 - 2 MR
 // (52 at 5 levels). 0: OW = 64 - 2 levels (54 at 5 levels: fewer redundant columns but 215 vs
@@ -281,8 +301,12 @@ struct TbGeom {
     static constexpr int OW = TEA_TB_GEOM == 0 ? kStrip - 2 * NL
                               : (TEA_TB_GEOM == 2 ? 48 : kStrip - 2 * MR);
     static_assert(SH >= NL && SH + OW <= kStrip - NL && OW % 2 == 0, "strip geometry");
-    static constexpr int D = 8;  // TMEM ring depth (rows k-NL..k fit for NL <= 6); a power of
-                                 // two so slots are (head - t) & 7
+    // TMEM ring depth: rows k-NL..k are live (NL + 1 slots). NL <= 5: 6 slots and the row
+    // loop unrolled by 6 = 2 x the window period 3, so every slot index of the unrolled body
+    // is a compile-time constant (no per-row address arithmetic or R2UR); NL = 6: 8 slots,
+    // unrolled by 3 (TEA_TB_RING6 0: always 8 and 3, round 1)
+    static constexpr int D = (TEA_TB_RING6 && NL <= 5) ? 6 : 8;
+    static constexpr int UNR = D == 6 ? 6 : 3;
 };
 
 #ifndef TEA_TB_MINB
@@ -399,7 +423,9 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     double dot0 = 0.0, dot1 = 0.0, dot2 = 0.0;  // r.z, r.r (LAST); z.(A z) (POST)
 
     const int kbeg = kt0 - NL, kend = kt1 + NL;
-    long long orow = (long long)kbeg * pitch + jA;  // offset of (jA, k); running, no k*pitch
+    // offset of (jA, k), running (no k*pitch); 32-bit: the host runs the passes only on
+    // fields of < 2^31 elements (tb_fits), so every address is one IMAD.WIDE
+    int orow = kbeg * pitch + jA;
     // Input rows are staged P rows ahead by cp.async into per-thread shared-memory slots
     // (each thread copies and later reads back only its own 16 B per stream, so no
     // barriers; slots the thread never fills stay zero): P rows of bytes in flight per
@@ -410,7 +436,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     for (int sl = 0; sl < NSL; ++sl)
 #pragma unroll
         for (int q = 0; q < kTbNS; ++q) cpa[sl][q][threadIdx.x] = z0;
-    auto issue = [&](long long o, int sl) {
+    auto issue = [&](int o, int sl) {
         if (ld_ok) {
             if (PRE) {  // z_s, p_old, r, g, u
                 cp16(&cpa[sl][0][threadIdx.x], zin1 + o);
@@ -433,7 +459,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
 #pragma unroll
     for (int i = 0; i < P; ++i) {
         if (kt0 < kt1 && kbeg + i < kend)
-            issue(orow + (long long)i * pitch, i);
+            issue(orow + i * pitch, i);
         else
             cp_commit();
     }
@@ -443,9 +469,9 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     double2 gprev = z0;   // KG: g of the previous input row (row kbeg-1's only feeds the
                           // pipeline-fill rows every pass discards)
     const double hrx = a.hrx, hry = a.hry;
-    constexpr int UNR = FIRST ? kTbUnroll : kTbUnrollL;
+    constexpr int UNR = G::UNR;
 #pragma unroll(UNR)
-    for (int k = kbeg; k < kend; ++k, orow += pitch, head = (head + 1) & (D - 1)) {
+    for (int k = kbeg; k < kend; ++k, orow += pitch, head = head + 1 == D ? 0 : head + 1) {
         cp_wait<P - 1>();  // row k's group (the oldest outstanding) has landed
         double2 X = cpa[cs][0][threadIdx.x];
         double2 KX, KY;
@@ -478,7 +504,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             // row k+P goes into the slot row k-1 used (read a full iteration ago)
             const int ns = cs == 0 ? P : cs - 1;
             if (kt0 < kt1 && k + P < kend)
-                issue(orow + (long long)P * pitch, ns);
+                issue(orow + P * pitch, ns);
             else
                 cp_commit();
             cs = cs == P ? 0 : cs + 1;
@@ -505,7 +531,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         tm_wait_st();
         tm_st12(tm + 16u * head, KX, KY, rk);
         TmRow tmA;
-        tm_ld12(tm + 16u * ((head - 1) & (D - 1)), tmA);  // row k-1: level 1's operands
+        tm_ld12(tm + 16u * ((head + D - 1) % D), tmA);  // row k-1: level 1's operands
         tm_wait_ld(tmA);
         double2 s_kx = tm_get(tmA, 0), s_ky = tm_get(tmA, 1), s_r = tm_get(tmA, 2), kyn = KY;
         // Row k-1 is completed now that its top faces (row k's Ky) are known: the diagonal
@@ -517,7 +543,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         double2 s_d;
         s_d.x = 1.0 + (s_kx.x + s_kx.y) + (s_ky.x + KY.x);
         s_d.y = 1.0 + (s_kx.y + kxE) + (s_ky.y + KY.y);
-        tm_st4(tm + 16u * ((head - 1) & (D - 1)) + 12u, s_d);
+        tm_st4(tm + 16u * ((head + D - 1) % D) + 12u, s_d);
         const double2 z2row = z2prev;  // z_{i-2} of row k-1
         if (!FIRST) z2prev = Z2;
         W[0][0] = W[0][1];
@@ -528,7 +554,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             const int q = k - t;
             // issue the next level's slot (row q-1) before computing this one
             TmRow tmB;
-            if (t < NL) tm_ld16(tm + 16u * ((head - t - 1) & (D - 1)), tmB);
+            if (t < NL) tm_ld16(tm + 16u * ((head + 2 * D - t - 1) % D), tmB);
             const double2 kx = s_kx, kyc = s_ky, rq = s_r;
             const double2 xm = W[t - 1][0], xc = W[t - 1][1], xp = W[t - 1][2];
             const double2 dg = s_d;
@@ -550,14 +576,23 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                 // w = A p; r' = r - alpha w = r + alpha (sum_f K_f p_f - d p)
                 zn.x = fma(alpha, fma(kyn.x, xp.x, nb.x), rq.x);
                 zn.y = fma(alpha, fma(kyn.y, xp.y, nb.y), rq.y);
-                tm_st4(tm + 16u * ((head - 1) & (D - 1)) + 8u, zn);  // row q's r is now r'
+                tm_st4(tm + 16u * ((head + D - 1) % D) + 8u, zn);  // row q's r is now r'
                 if (rowout) st2m(rout + (orow - pitch), zn, oA, oB);
             } else if (POST && t == NL) {
-                // q = A z_s at row q (xc = z_s): z_s . q over the owned cells
+                // q = A z_s at row q (xc = z_s): z_s . q, and r . z_s, r . r of the same row
+                // (rq), over the owned cells
                 if (rowout && q >= Dd.k0 && q < Dd.k1) {
                     const double mx = fma(kyn.x, xp.x, nb.x), my = fma(kyn.y, xp.y, nb.y);
-                    if (dA) dot2 -= xc.x * mx;
-                    if (dB) dot2 -= xc.y * my;
+                    if (dA) {
+                        dot2 -= xc.x * mx;
+                        dot0 += rq.x * xc.x;
+                        dot1 += rq.x * rq.x;
+                    }
+                    if (dB) {
+                        dot2 -= xc.y * my;
+                        dot0 += rq.y * xc.y;
+                        dot1 += rq.y * rq.y;
+                    }
                 }
             } else {
                 // Chebyshev step j of this pass (DESIGN.md §4.3 recurrence):
@@ -588,7 +623,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                 if (j == M - 1 && !LAST && rowout) st2m(zoutA + (orow - t * pitch), zn, oA, oB);
                 if (j == M && rowout) {
                     st2m(zoutB + (orow - t * pitch), zn, oA, oB);
-                    if (LAST && q >= Dd.k0 && q < Dd.k1) {
+                    if (LAST && !POST && q >= Dd.k0 && q < Dd.k1) {
                         if (dA) {
                             dot0 += rq.x * zn.x;
                             dot1 += rq.x * rq.x;
