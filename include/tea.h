@@ -38,7 +38,10 @@ typedef enum {
     TEA_NOT_CONVERGED = 1,
     TEA_ERR_ARG = -1,       /* bad argument: sizes, decomposition, depth, workspace   */
     TEA_ERR_CUDA = -2,      /* CUDA runtime error (message in tea_last_error)          */
-    TEA_ERR_NCCL = -3,      /* NCCL error                                              */
+    TEA_ERR_NCCL = -3,      /* NCCL error; in multi-process runs also an asynchronous
+                               NCCL error or no completion within TEA_NCCL_TIMEOUT_S seconds
+                               (environment, default 600) -- a dead or stalled peer: the
+                               host waits poll ncclCommGetAsyncError and abort the comm  */
     TEA_ERR_BREAKDOWN = -4, /* p.w <= 0, non-finite scalar, or bad eigen-estimate      */
     TEA_ERR_STATE = -5      /* call out of order / context already failed             */
 } tea_status;

@@ -44,10 +44,18 @@ def stale() -> bool:
     return any(os.path.getmtime(f) > t for f in deps())
 
 
+def nvtx_include() -> str:
+    for p in sys.path:
+        d = os.path.join(p, "nvidia", "nvtx", "include")
+        if os.path.exists(os.path.join(d, "nvtx3", "nvToolsExt.h")):
+            return d
+    return "/usr/local/cuda/include"  # the toolkit ships nvtx3 too
+
+
 def nvcc_cmd(out: str, extra=()):
     nccl = nccl_dir()
     return ["nvcc", "-O3", "-std=c++17", *ARCH, "-lineinfo", "-Xcompiler", "-fPIC", "-shared",
-            "-I" + INCLUDE, "-I" + os.path.join(nccl, "include"),
+            "-I" + INCLUDE, "-I" + os.path.join(nccl, "include"), "-I" + nvtx_include(),
             "-L" + os.path.join(nccl, "lib"), "-l:libnccl.so.2",
             "-Xlinker", "-rpath," + os.path.join(nccl, "lib"),
             *extra, "-o", out, *sources()]

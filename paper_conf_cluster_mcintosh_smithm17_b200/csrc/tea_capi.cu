@@ -9,9 +9,13 @@
 #include "tea_internal.h"
 
 #include <nccl.h>
+#include <nvtx3/nvToolsExt.h>
 
 #include <algorithm>
+#include <chrono>
 #include <cmath>
+#include <cstdlib>
+#include <thread>
 #include <cstdarg>
 #include <cstdio>
 #include <cstring>
@@ -191,6 +195,51 @@ struct TeaError {
                  ncclGetErrorString(r_));                                               \
     } while (0)
 
+// Host wait for the library stream. Multi-process runs poll instead of blocking: a peer that
+// died or an NCCL error would otherwise hang the rank forever (SURVEY §5 failure detection).
+// ncclCommGetAsyncError is checked every poll; after TEA_NCCL_TIMEOUT_S seconds (default
+// 600) without completion, or on an NCCL error, the communicator is aborted and the call
+// fails with TEA_ERR_NCCL.
+void wait_stream(tea_ctx *c) {
+    if (c->nranks <= 1 || !c->comm) {
+        CK(cudaStreamSynchronize(c->stream));
+        return;
+    }
+    static const double timeout_s = [] {
+        const char *e = std::getenv("TEA_NCCL_TIMEOUT_S");
+        const double v = e ? std::atof(e) : 0.0;
+        return v > 0.0 ? v : 600.0;
+    }();
+    const auto t0 = std::chrono::steady_clock::now();
+    for (long long n = 0;; ++n) {
+        const cudaError_t q = cudaStreamQuery(c->stream);
+        if (q == cudaSuccess) return;
+        if (q != cudaErrorNotReady) CK(q);
+        ncclResult_t ar = ncclSuccess;
+        NK(ncclCommGetAsyncError(c->comm, &ar));
+        const double dt =
+            std::chrono::duration<double>(std::chrono::steady_clock::now() - t0).count();
+        if (ar != ncclSuccess && ar != ncclInProgress) {
+            ncclCommAbort(c->comm);
+            c->comm = nullptr;
+            fail(TEA_ERR_NCCL, "NCCL async error: %s", ncclGetErrorString(ar));
+        }
+        if (dt > timeout_s) {
+            ncclCommAbort(c->comm);
+            c->comm = nullptr;
+            fail(TEA_ERR_NCCL, "no completion after %.0f s (TEA_NCCL_TIMEOUT_S): a peer rank "
+                 "is gone or stalled; communicator aborted", dt);
+        }
+        if (n > 64) std::this_thread::sleep_for(std::chrono::microseconds(n > 4096 ? 200 : 20));
+    }
+}
+
+// NVTX phase ranges (nvtx3, header only: no-ops unless a tool such as nsys is attached)
+struct Nvtx {
+    explicit Nvtx(const char *name) { nvtxRangePushA(name); }
+    ~Nvtx() { nvtxRangePop(); }
+};
+
 KArgs kargs(tea_ctx *c, const BlockCtx &b, bool set_cond = false) {
     KArgs a;
     a.pitch = b.L.pitch;
@@ -263,7 +312,7 @@ void K(tea_ctx *c, int kid, double bytes, F &&f) {
 
 void resolve_profile(tea_ctx *c) {
     if (!c->profiling) return;
-    CK(cudaStreamSynchronize(c->stream));
+    wait_stream(c);
     for (auto &p : c->pending) {
         float ms = 0.f;
         CK(cudaEventElapsedTime(&ms, p.a, p.b));
@@ -321,6 +370,7 @@ Launch plan_pw(tea_ctx *c, const BlockCtx &b, const Region &R) {
 // Combine the block-local sums of slots [first, first+n) (0 pw, 1 gam, 2 rr) into
 // the global sums on every local block and across ranks.
 void reduce(tea_ctx *c, int first, int n) {
+    Nvtx nv_("tea reduce");
     const int nb = (int)c->blocks.size();
     if (nb > 1) {
         std::vector<Scalars *> L;
@@ -343,6 +393,7 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
     const cudaStream_t st = xs ? xs : c->stream;
     const int nb = (int)c->blocks.size();
     if (c->px * c->py == 1) return;
+    Nvtx nv_("tea halo exchange");
     const int nf = (int)fids_per_block_field.size();
     for (auto &b : c->blocks) {
         const XPlan &x = b.xp[kind];
@@ -978,7 +1029,7 @@ void body_stat(tea_ctx *c, bool cheb, int par, bool sets_cond) {
 void read_state(tea_ctx *c) {
     CK(cudaMemcpyAsync(c->hS, c->blocks[0].S, offsetof(Scalars, cheb_a),
                        cudaMemcpyDeviceToHost, c->stream));
-    CK(cudaStreamSynchronize(c->stream));
+    wait_stream(c);
     resolve_profile(c);
 }
 
@@ -1150,6 +1201,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
             launch_scalars(kargs(c, b), SC_BEGIN, eps, lim1, max_iters, c->opts.eig_margin_lo,
                            c->opts.eig_margin_hi, c->stream);
         });
+    Nvtx nv_solve("tea_solve");
     const bool persist = use_persist(c, method);
     int ds = DS_RUNNING;
     bool phase2 = false;
@@ -1208,6 +1260,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
 
     // ---- phase 1: CG (or the CPPCG presteps), or block-Jacobi PCG
     if (!c->hS->done) {
+        Nvtx nv_("tea phase 1 (CG / presteps)");
         if (method == TEA_BJCG)
             run_loop(c, 3, lim1, [&](int par, bool sc) { body_bj(c, par, sc); });
         else if (method == TEA_CG1)
@@ -1238,6 +1291,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
                                    cudaMemcpyDeviceToDevice, c->stream));
         ds = c->hS->status;
     } else if (phase2) {
+        Nvtx nv_("tea phase 2 (eigen-estimate, restart, PCG)");
         // ---- eigen-estimate, coefficients, restart z = B(A) r, p = z
         for (auto &b : c->blocks)
             K(c, TEA_K_EIG, 0.0, [&] { launch_eig_setup(kargs(c, b), s, c->stream); });
@@ -1298,7 +1352,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
     CK(cudaEventRecord(c->ev_t1, c->stream));
     CK(cudaEventRecord(c->ev_in, c->stream));
     CK(cudaStreamWaitEvent(c->user_stream, c->ev_in, 0));
-    CK(cudaStreamSynchronize(c->stream));
+    wait_stream(c);
     float ms = 0.f;
     CK(cudaEventElapsedTime(&ms, c->ev_t0, c->ev_t1));
     const Scalars &h = *c->hS;
