@@ -412,7 +412,8 @@ def run_gpu(args):
               "cppcg1": tea.CPPCG1, "cppcg1f": tea.CPPCG1F}[args.method]
     cells = args.n * args.n * max(args.nz, 1)
     t = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
-                tile_rows=args.tile_rows, tb_steps=args.tb_steps, loop_mode=args.loop_mode,
+                tile_rows=args.tile_rows, tb_steps=args.tb_steps, tb_rows=args.tb_rows,
+                loop_mode=args.loop_mode,
                 persist=args.persist, overlap=args.overlap, kform=args.kform,
                 trace=not args.no_trace)
     stream = t.stream
@@ -568,6 +569,7 @@ def main():
                     help="PXxPY: run the px x py decomposition inside ONE process on one GPU "
                          "(the multi-GPU code path with device-copy halos instead of NCCL)")
     ap.add_argument("--tile-rows", type=int, default=0)
+    ap.add_argument("--tb-rows", type=int, default=0, help="output rows per fused-pass tile (0 auto)")
     ap.add_argument("--persist", type=int, default=0,
                     help="whole solve in one cooperative launch: 1 on, 0 (auto) or -1 off "
                          "(tea_opts.persist)")

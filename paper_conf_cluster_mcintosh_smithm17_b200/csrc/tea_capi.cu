@@ -678,6 +678,10 @@ struct ChainX {
     bool pre = false, post = false;
     bool even = false;  // CPPCG1F on one block: the pass split of chain_passes(.., true)
     int zs = -1, pin = -1, pout = -1;
+    // CPPCG with neighbour blocks, update fused into the first pass: exchange (r_old, w) at
+    // depth d -- it needs no alpha, so it is issued before (and with overlap: concurrently
+    // with) the p.w reduction, which this chain then performs
+    bool xw = false;
 };
 
 // Passes of a chain. CPPCG1F on one block (pre and post): an even number of passes >= 2, so
@@ -713,15 +717,19 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
     const bool want = c->opts.overlap > 0 || (c->opts.overlap == 0 && c->nranks > 1);
     const bool ovl = blocks && c->xstream && want && !c->profiling && passes.size() > 1;
     if (blocks) {
+        // depth d >= s + 1, with corners: r, or (r_old, w) for the fused update
+        const int kind = x.xw ? X_Z2 : X_RD;
+        const std::vector<int> fields = x.xw ? std::vector<int>{rin, F_W} : std::vector<int>{rin};
         if (ovl) {
             CK(cudaEventRecord(c->ev_fork, c->stream));
             CK(cudaStreamWaitEvent(c->xstream, c->ev_fork, 0));
-            exchange(c, X_RD, {rin}, c->xstream);  // depth d >= s + 1, with corners
+            exchange(c, kind, fields, c->xstream);
             CK(cudaEventRecord(c->ev_join, c->xstream));
         } else {
-            exchange(c, X_RD, {rin});
+            exchange(c, kind, fields);
         }
     }
+    if (x.xw) reduce(c, 0, 1);  // p.w -> alpha, while the exchange is in flight
     int step0 = 1, after = s;
     const int r = (fused || f1) ? rout : rin;
     for (size_t p = 0; p < passes.size(); ++p) {
@@ -863,6 +871,15 @@ void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
             launch_spmv(kargs(c, b), L, R, b.f[zs], b.f[F_P0 + par], b.f[F_P1 - par],
                         b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
         });
+    }
+    if (!fused && use_tb(c, s)) {
+        // blocks with the fused passes: r -= alpha w in the first pass on the extended
+        // bounds, from (r_old, w) exchanged at depth d -- no separate update kernel (its 3
+        // streams), and the exchange overlaps the p.w reduction
+        ChainX x;
+        x.xw = true;
+        cheb_chain_tb(c, s, false, true, F_R0 + par, F_R1 - par, sets_cond, true, x);
+        return;
     }
     reduce(c, 0, 1);
     if (fused) {

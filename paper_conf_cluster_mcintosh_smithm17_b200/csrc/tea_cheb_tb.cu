@@ -24,6 +24,9 @@
 // neighbour blocks (matrix powers across blocks).
 #include "tea_internal.h"
 
+#include <algorithm>
+#include <cstdio>
+#include <cstdlib>
 #include <mutex>
 
 namespace tea {
@@ -719,6 +722,8 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
     if (!(attr.load() & bit)) {
         cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST, KG, PRE, POST>,
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST, KG, PRE, POST>,
+                             cudaFuncAttributePreferredSharedMemoryCarveout, 100);
         attr.fetch_or(bit);
     }
     k_cheb_tb<M, FIRST, FUSE, LAST, KG, PRE, POST><<<grid, kTbT, smem, st>>>(
@@ -774,48 +779,72 @@ static void tb_dispatch(const KArgs &a, const Region &R, const Region &Dd, int t
 
 int tb_max_steps() { return 5; }
 
-// Rows per CTA tile: a CTA costs ~ (ty + 2 NL) row-iterations (pipeline fill/drain), all
-// CTAs are alike, so a launch costs ~ waves x (ty + 2 NL) with waves = ceil(ctas / slots).
-// Pick ty minimising that (slots = SMs x resident CTAs per SM of a pass with NL levels).
+// Rows per CTA tile: a CTA costs ~ (ty + 2 NL) row-iterations (pipeline fill/drain); an SM
+// holding n CTAs of a wave runs them at a rate that grows with n but saturates (the passes
+// are latency-bound with few warps, issue-bound with 3 CTAs), modelled as n / (n + 1/2): a
+// launch costs waves x (ty + 2 NL) x (n + 1/2). This keeps 4096^2's full wave of 187-row
+// tiles and picks fewer, taller tiles where a full wave would make them short (2048 x 1024
+// blocks: 24-row tiles at 3 CTAs per SM 393 / 460 us vs 32-row tiles at ~2.2 per SM 360 /
+// 385 us per 5 timesteps, profiles/r02_blocks_ab.txt). The occupancy is computed from the
+// kernel's registers and shared memory: cudaOccupancyMaxActiveBlocksPerMultiprocessor reports
+// 1 CTA per SM for these kernels while 3 are resident (ncu), which made every earlier plan a
+// "3-wave" one.
 int tb_auto_rows(int NL, int width, int height) {
     static std::atomic<int> slot_cache[kMaxDev][8];
+    static std::atomic<int> sm_cache[kMaxDev];
     NL = NL < 1 ? 1 : (NL > 6 ? 6 : NL);
     const int dev = tea_device();
     int slots = slot_cache[dev][NL].load();
     if (!slots) {
-        int nsm = 148, per = 0;
+        int nsm = 148, per = 0, smem_sm = 0;
         cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, dev);
+        cudaDeviceGetAttribute(&smem_sm, cudaDevAttrMaxSharedMemoryPerMultiprocessor, dev);
         const size_t smem = tb_smem_bytes();
         cudaError_t e = cudaSuccess;
+        // resident CTAs per SM from the kernel's registers and shared memory (the occupancy
+        // API reports 1 for these kernels, round 2 probe -- ncu shows ~3 resident), capped
+        // by the TMEM columns (512 per SM, 128 per CTA)
+        cudaFuncAttributes fa{};
         switch (NL) {
 #define OCC(m, POST)                                                                             \
     case (m + (POST ? 1 : 0)):                                                                   \
-        cudaFuncSetAttribute(k_cheb_tb<m, false, false, true, true, false, POST>,                \
-                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);            \
-        e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(                                       \
-            &per, k_cheb_tb<m, false, false, true, true, false, POST>, kTbT, smem);              \
+        e = cudaFuncGetAttributes(&fa, k_cheb_tb<m, false, false, true, true, false, POST>);     \
         break;
             OCC(1, false) OCC(2, false) OCC(3, false) OCC(4, false) OCC(5, false) OCC(5, true)
 #undef OCC
         }
+        if (e == cudaSuccess && fa.numRegs > 0) {
+            const int regs_cta = ((fa.numRegs * 32 + 255) / 256 * 256) * (kTbT / 32);
+            const int by_regs = 65536 / regs_cta;
+            const int by_smem = smem_sm / (int)(smem + fa.sharedSizeBytes + 1024);
+            per = std::min(std::min(by_regs, by_smem), 512 / kTmCols);
+        }
         if (e != cudaSuccess || per < 1) per = 1;
         slots = nsm * per;
         slot_cache[dev][NL].store(slots);
+        if (std::getenv("TEA_DEBUG_PLAN"))
+            fprintf(stderr, "tea: fused pass NL=%d: %d CTAs/SM (%s), %d SMs\n", NL, per,
+                    cudaGetErrorString(e), nsm);
+        sm_cache[dev].store(nsm);
     }
+    const int nsm = std::max(1, sm_cache[dev].load());
     const int ow = tb_out_cols(NL);
     const int gx = (width + ow - 1) / ow;
-    int best = height, bestc = 0x7fffffff;
-    for (int w = 1; w <= 256; ++w) {
-        const int tiles = (int)((long long)slots * w / gx);
-        if (tiles < 1) continue;
-        const int ty = (height + tiles - 1) / tiles;
-        const int waves = (int)(((long long)gx * ((height + ty - 1) / ty) + slots - 1) / slots);
-        const long long cost = (long long)waves * (ty + 2 * NL);
-        if (cost < bestc) {
-            bestc = (int)cost;
+    int best = height;
+    double bestc = 1e300;
+    // tiles of at most 512 rows: taller ones leave the scheduler no CTAs to balance the SMs
+    // with (16384^2: one wave of 3277-row tiles 2541 us vs waves of ~1261-row tiles 2382 us
+    // per first pass, profiles/r02_blocks_ab.txt)
+    for (int ty = std::max(1, height / 4096); ty <= std::min(height, 512); ++ty) {
+        const long long ctas = (long long)gx * ((height + ty - 1) / ty);
+        const long long waves = (ctas + slots - 1) / slots;
+        const double per_sm = waves > 1 ? (double)slots / nsm
+                                         : std::max(1.0, (double)(ctas - (waves - 1) * slots) / nsm);
+        const double cost = (double)waves * (ty + 2 * NL) * (per_sm + 0.5);
+        if (cost < bestc - 1e-9) {
+            bestc = cost;
             best = ty;
         }
-        if (ty <= 2 * NL) break;
     }
     return best < 1 ? 1 : best;
 }
