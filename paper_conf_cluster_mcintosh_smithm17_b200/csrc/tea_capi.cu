@@ -37,7 +37,8 @@ constexpr int kOpp[kNDir] = {1, 0, 3, 2, 7, 6, 5, 4};
 inline size_t round_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
 
 // exchange kinds
-enum { X_R1 = 0, X_RD, X_Z2, X_Z1, X_U1, X_COUNT };
+// X_ZD1: z_s at depth d + 1 (CPPCG1F on blocks, exchanged while its one reduction is in flight)
+enum { X_R1 = 0, X_RD, X_Z2, X_Z1, X_U1, X_ZD1, X_COUNT };
 
 struct XPlan {
     int nf = 0, depth = 0;
@@ -478,7 +479,7 @@ void build_xplans(tea_ctx *c, BlockCtx &b, int *d_boxes_base) {
         int nf, dep;
         bool corners;
     } kinds[X_COUNT] = {{1, 1, false}, {1, c->d, c->d > 1}, {2, c->d, c->d > 1},
-                        {1, 1, false}, {1, 1, false}};
+                        {1, 1, false}, {1, 1, false}, {1, c->d + 1, true}};
     std::vector<int> host;
     int *dptr = d_boxes_base;
     for (int kd = 0; kd < X_COUNT; ++kd) {
@@ -682,6 +683,10 @@ struct ChainX {
     // depth d -- it needs no alpha, so it is issued before (and with overlap: concurrently
     // with) the p.w reduction, which this chain then performs
     bool xw = false;
+    // CPPCG1F with neighbour blocks: r is already valid on ext(d) (no exchange before the
+    // passes); after the last pass z_s is exchanged at depth d + 1 while the chain's one
+    // reduction [z.q, r.z, r.r] is in flight
+    bool noexch = false, xz = false;
 };
 
 // Passes of a chain. CPPCG1F on one block (pre and post): an even number of passes >= 2, so
@@ -715,8 +720,9 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
     // follows the exchange. The first pass must not be the last (its dot products are one
     // grid reduction); profiling keeps every launch on the compute stream.
     const bool want = c->opts.overlap > 0 || (c->opts.overlap == 0 && c->nranks > 1);
-    const bool ovl = blocks && c->xstream && want && !c->profiling && passes.size() > 1;
-    if (blocks) {
+    const bool ovl = blocks && !x.noexch && c->xstream && want && !c->profiling &&
+                     passes.size() > 1;
+    if (blocks && !x.noexch) {
         // depth d >= s + 1, with corners: r, or (r_old, w) for the fused update
         const int kind = x.xw ? X_Z2 : X_RD;
         const std::vector<int> fields = x.xw ? std::vector<int>{rin, F_W} : std::vector<int>{rin};
@@ -817,8 +823,27 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
         }
         step0 += M;
     }
+    const int zs_out = pairB[(passes.size() - 1) % 2];
+    if (x.xz && blocks) {
+        // the next outer update runs on ext(d) and needs z_s on ext(d + 1): exchange it while
+        // the single reduction is in flight ("the communications can be
+        // overlapped")
+        const bool ovx = c->xstream && want && !c->profiling;
+        if (ovx) {
+            CK(cudaEventRecord(c->ev_fork, c->stream));
+            CK(cudaStreamWaitEvent(c->xstream, c->ev_fork, 0));
+            exchange(c, X_ZD1, {zs_out}, c->xstream);
+            CK(cudaEventRecord(c->ev_join, c->xstream));
+            if (reduce_dots) reduce(c, 0, 3);
+            CK(cudaStreamWaitEvent(c->stream, c->ev_join, 0));
+        } else {
+            exchange(c, X_ZD1, {zs_out});
+            if (reduce_dots) reduce(c, 0, 3);
+        }
+        return zs_out;
+    }
     if (reduce_dots) reduce(c, x.post ? 0 : 1, x.post ? 3 : 2);
-    return pairB[(passes.size() - 1) % 2];
+    return zs_out;
 }
 
 
@@ -1001,17 +1026,24 @@ void body_pcg1f(tea_ctx *c, int s, int par, bool sets_cond) {
         cheb_chain_tb(c, s, false, false, F_R0 + par, F_R1 - par, sets_cond, true, x);
         return;
     }
+    const bool tb = use_tb1f(c, s);
     for (auto &b : c->blocks) {
-        Region R = b.owned();
+        // fused passes across blocks: the update runs on ext(d) (z_s arrived at depth d + 1
+        // with the last reduction; p is kept valid on ext(d + 1) by this kernel's ring), so r
+        // needs no exchange at all; else on the owned cells, r exchanged by the chain
+        Region R = tb ? b.ext(c->d) : b.owned();
         Launch L = plan_spmv(c, b, R);
         K(c, TEA_K_UPDATE, sbytes(b, 7 + kstreams(c, b)), [&] {  // z, p, r, u -> p, r, u
-            launch_cg1f_pre(kargs(c, b), L, R, b.f[zs], b.f[F_P0 + par], b.f[F_P1 - par],
-                            b.f[F_R0], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
+            launch_cg1f_pre(kargs(c, b), L, R, b.owned(), b.f[zs], b.f[F_P0 + par],
+                            b.f[F_P1 - par], b.f[F_R0], b.f[F_U], b.f[F_KX], b.f[F_KY],
+                            c->stream);
         });
     }
-    if (use_tb1f(c, s)) {
+    if (tb) {
         ChainX x;
         x.post = true;
+        x.noexch = true;
+        x.xz = true;
         cheb_chain_tb(c, s, false, false, F_R0, F_R0, sets_cond, true, x);
         return;
     }
@@ -1321,6 +1353,7 @@ tea_status solve_impl(tea_ctx *c, tea_method method, double eps, int max_iters, 
                 ChainX x;
                 x.post = true;
                 x.even = single_block(c);
+                x.xz = !single_block(c);  // blocks: z_s to depth d + 1 for the first update
                 cheb_chain_tb(c, s, true, false, F_R0, F_R0, false, true, x);
             } else {
                 chain(c, s, true, false, F_R0, F_R0, false, false);

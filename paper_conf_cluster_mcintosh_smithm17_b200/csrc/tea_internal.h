@@ -252,9 +252,10 @@ void launch_cg1_w(const KArgs &a, const Launch &L, const Region &R, const double
 
 // Single-reduction CPPCG, fused form (CPPCG1F): the outer update as one stencil pass
 // (p = z + b p on R + ring, w = A p, r -= a w, u += a p), where the fused passes do not.
-void launch_cg1f_pre(const KArgs &a, const Launch &L, const Region &R, const double *z,
-                     const double *pin, double *pout, double *r, double *u, const double *kx,
-                     const double *ky, cudaStream_t st);
+// r on R (may be extended toward neighbour blocks), u on D (the owned cells)
+void launch_cg1f_pre(const KArgs &a, const Launch &L, const Region &R, const Region &D,
+                     const double *z, const double *pin, double *pout, double *r, double *u,
+                     const double *kx, const double *ky, cudaStream_t st);
 
 // Temporally blocked Chebyshev passes (tea_cheb_tb.cu).
 constexpr int kTbMaxSteps = 5;

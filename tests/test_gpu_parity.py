@@ -818,3 +818,23 @@ def test_cppcg1f_loop_modes_identical(tea, loop_mode):
     u, st = gpu_run(tea, deck, loop_mode=loop_mode, check_interval=6, **kw)
     assert st[0]["iterations"] == st_ref[0]["iterations"]
     assert np.array_equal(u, ref)
+
+
+@pytest.mark.parametrize("nx,ny,px,py,d", [(240, 200, 2, 2, 11), (201, 143, 3, 2, 12), (150, 96, 1, 3, 6)])
+@pytest.mark.parametrize("loop_mode", [0, 2])
+def test_cppcg1f_blocks_overlap_bitwise(tea, ora, nx, ny, px, py, d, loop_mode):
+    """CPPCG1F across blocks with the fused passes: the outer update on ext(d), z_s exchanged
+    at depth d + 1 while the one reduction is in flight (on the second stream with overlap on,
+    NEXT-2 / P:L817-821): bitwise the same as without the overlap, and the oracle's solution."""
+    deck = deck_of("random", nx, ny, seed=nx + ny, dt=0.04)
+    s = d - 1
+    kw = dict(method=7, eps=0.0, max_iters=30 + 5, inner_steps=s, tb_steps=5, loop_mode=loop_mode,
+              dist=dict(px=px, py=py, halo_depth=d, nranks=1))
+    u_a, st_a = gpu_run(tea, deck, overlap=1, **kw)
+    u_b, st_b = gpu_run(tea, deck, overlap=-1, **kw)
+    assert st_a[0]["iterations"] == st_b[0]["iterations"] == 35
+    assert np.array_equal(u_a, u_b)
+    assert st_a[0]["rnorm"] == st_b[0]["rnorm"]
+    u_o, st_o, _ = ora.run(deck, steps=1, method=7, eps=0.0, max_iters=35, inner_steps=s)
+    assert iter_err(u_a, u_o, "random") <= 1e-12
+    assert st_a[0]["rnorm"] == pytest.approx(st_o[0]["rnorm"], rel=1e-9)
