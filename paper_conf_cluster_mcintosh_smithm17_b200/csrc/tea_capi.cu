@@ -744,7 +744,8 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
         const bool first = p == 0, last = p + 1 == passes.size();
         const bool fu = fused && first;
         const bool pre = x.pre && first, post = x.post && last;
-        const int levels = M + (pre ? 1 : 0) + (post ? 1 : 0);
+        // (post with odd M: z.(A z) from faces, no extra level -- tea_cheb_tb.cu POSTF)
+        const int levels = M + (pre ? 1 : 0) + ((post && (M + (pre ? 1 : 0)) % 2 == 0) ? 1 : 0);
         const int o = p % 2, in = (p + 1) % 2;
         // the regions this pass is launched on, per block: the whole (extended) region, or
         // for the overlapped first pass the halo-free interior now and the frame after the

@@ -338,7 +338,12 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
               const double *__restrict__ Ky, const double *__restrict__ pin,
               double *__restrict__ pout, double *__restrict__ uio, KArgs a, Region R,
               Region Dd, int ty, int jlim, int step0, int restart) {
-    constexpr int NL = M + (PRE ? 1 : 0) + (POST ? 1 : 0);  // stencil levels
+    // POST with an odd level count: z.(A z) = sum z^2 + sum_faces K_f (z_i - z_j)^2 from the
+    // last step's output itself (each face counted by its west / south cell, as that cell's
+    // east / north face; an odd level count leaves the spare valid column east of the output
+    // columns) -- no extra stencil level. Even: a stencil level q = A z_s after the last step.
+    constexpr bool POSTF = POST && ((M + (PRE ? 1 : 0)) % 2 == 1);
+    constexpr int NL = M + (PRE ? 1 : 0) + ((POST && !POSTF) ? 1 : 0);  // stencil levels
     constexpr int T0 = PRE ? 2 : 1;                         // level of the first Chebyshev step
     using G = TbGeom<NL>;
     constexpr int D = G::D;
@@ -425,7 +430,9 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     for (int t = 0; t < NL; ++t) W[t][0] = W[t][1] = W[t][2] = z0;
     double dot0 = 0.0, dot1 = 0.0, dot2 = 0.0;  // r.z, r.r (LAST); z.(A z) (POST)
 
-    const int kbeg = kt0 - NL, kend = kt1 + NL;
+    // (POSTF: one more row-iteration, for the north face of the tile's last row)
+    const int kbeg = kt0 - NL, kend = kt1 + NL + (POSTF ? 1 : 0);
+    double2 zsp = z0;  // POSTF: the last step's previous row
     // offset of (jA, k), running (no k*pitch); 32-bit: the host runs the passes only on
     // fields of < 2^31 elements (tb_fits), so every address is one IMAD.WIDE
     int orow = kbeg * pitch + jA;
@@ -581,7 +588,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                 zn.y = fma(alpha, fma(kyn.y, xp.y, nb.y), rq.y);
                 tm_st4(tm + 16u * ((head + D - 1) % D) + 8u, zn);  // row q's r is now r'
                 if (rowout) st2m(rout + (orow - pitch), zn, oA, oB);
-            } else if (POST && t == NL) {
+            } else if (POST && !POSTF && t == NL) {
                 // q = A z_s at row q (xc = z_s): z_s . q, and r . z_s, r . r of the same row
                 // (rq), over the owned cells
                 if (rowout && q >= Dd.k0 && q < Dd.k1) {
@@ -624,9 +631,27 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                 zn.x = fma(ca, fma(kyn.x, xp.x, nb.x), base.x);
                 zn.y = fma(ca, fma(kyn.y, xp.y, nb.y), base.y);
                 if (j == M - 1 && !LAST && rowout) st2m(zoutA + (orow - t * pitch), zn, oA, oB);
+                if (POSTF && j == M) {
+                    // z.(A z) by faces, each face from its west / south cell: this row's
+                    // z^2 and east faces, and the north face of the row below (kyc = Ky(q))
+                    const double zE = __shfl_down_sync(0xffffffffu, zn.x, 1);
+                    const double kE = __shfl_down_sync(0xffffffffu, kx.x, 1);
+                    if (rowout && q >= Dd.k0 && q < Dd.k1) {
+                        const double ea = zn.x - zn.y, eb = zn.y - zE;
+                        if (dA) dot2 += fma(kx.y * ea, ea, zn.x * zn.x);
+                        if (dB) dot2 += fma(kE * eb, eb, zn.y * zn.y);
+                    }
+                    const int qs = q - 1;
+                    if (qs >= kt0 && qs < kt1 && qs >= Dd.k0 && qs < Dd.k1) {
+                        const double na = zsp.x - zn.x, nb2 = zsp.y - zn.y;
+                        if (dA) dot2 += kyc.x * na * na;
+                        if (dB) dot2 += kyc.y * nb2 * nb2;
+                    }
+                    zsp = zn;
+                }
                 if (j == M && rowout) {
                     st2m(zoutB + (orow - t * pitch), zn, oA, oB);
-                    if (LAST && !POST && q >= Dd.k0 && q < Dd.k1) {
+                    if (LAST && !(POST && !POSTF) && q >= Dd.k0 && q < Dd.k1) {
                         if (dA) {
                             dot0 += rq.x * zn.x;
                             dot1 += rq.x * rq.x;
@@ -711,7 +736,7 @@ int tb_out_cols(int NL) {
 template <int M, bool FIRST, bool FUSE, bool LAST, bool KG, bool PRE, bool POST>
 static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty, int jlim,
                       int step0, bool restart, const TbArgs &f, cudaStream_t st) {
-    constexpr int NL = M + (PRE ? 1 : 0) + (POST ? 1 : 0);
+    constexpr int NL = M + (PRE ? 1 : 0) + ((POST && (M + (PRE ? 1 : 0)) % 2 == 0) ? 1 : 0);
     const int width = R.j1 - (R.j0 & (TEA_TB_GEOM == 2 ? ~3 : ~1));
     const int ow = tb_out_cols(NL);
     dim3 grid((width + ow - 1) / ow, (R.k1 - R.k0 + ty - 1) / ty);
