@@ -528,14 +528,47 @@ def run_gpu(args):
         "time_to_solution_s": ms * 1e-3 / args.steps,
         "iterations_per_step": iters / args.steps, "outer_per_step": outer / args.steps,
         "matvecs_per_s": matvecs / (ms * 1e-3),
-        # library-accounted algorithmic bytes (fused passes counted as
-        # what they move), per iteration from the profiled solve, over the timed region
+        # library-accounted algorithmic bytes of the launches timed in-graph (
+        # fused passes counted as what they move) over the timed region
         "hbm_gbs_model": roof["model_gbs_timed_region"] if roof else None,
         # the same work priced at one kernel per Chebyshev step (6 streams / step):
         # an "effective bandwidth" that exceeds the HBM peak when fusion saves bytes
         "hbm_gbs_unfused_equiv": model_bytes / (ms * 1e-3) / 1e9,
         "e2e": e2e, "gpu_launches": launches, "clocks": clocks, "roofline": roof,
     }
+    # the same workload by the single-reduction CPPCG in fused form (TEA_CPPCG1F, SURVEY NEXT-2:
+    # one reduction and two fused kernels per outer iteration), same steps and timing
+    if args.method == "cppcg" and not args.no_variants:
+        tv = tea.Tea(tea.mesh_of(deck), deck.density, deck.energy, deck.dt, dist=dist_kw,
+                     tile_rows=args.tile_rows, tb_steps=args.tb_steps, tb_rows=args.tb_rows,
+                     loop_mode=args.loop_mode, persist=args.persist, overlap=args.overlap,
+                     kform=args.kform, trace=not args.no_trace)
+        for _ in range(args.warmup):
+            tv.solve(tea.CPPCG1F, args.eps, args.max_iters, args.inner)
+        barrier()
+        if not args.no_trace:
+            tv.trace(reset=True)
+        v0 = torch.cuda.Event(enable_timing=True)
+        v1 = torch.cuda.Event(enable_timing=True)
+        v0.record(tv.stream)
+        vst = [tv.solve(tea.CPPCG1F, args.eps, args.max_iters, args.inner).stats
+               for _ in range(args.steps)]
+        v1.record(tv.stream)
+        v1.synchronize()
+        vms = max_over_ranks(v0.elapsed_time(v1))
+        vtr = [] if args.no_trace else tv.trace()
+        tv.close()
+        vcls = {}
+        for kname, bpl, n, kms in vtr:
+            e = vcls.setdefault(kname, [0.0, 0])
+            e[0] += kms
+            e[1] += n
+        line["variants"] = {"cppcg1f": {
+            "method": "single-reduction CPPCG, fused form (TEA_CPPCG1F)",
+            "value": sum(x["iterations"] for x in vst) / (vms * 1e-3), "unit": "iterations/s",
+            "ms_per_step": vms / args.steps,
+            "iterations_per_step": sum(x["iterations"] for x in vst) / args.steps,
+            "kernel_avg_us": {k: round(v[0] / max(v[1], 1) * 1e3, 1) for k, v in vcls.items()}}}
     if rank == 0 and world == 1 and not args.no_cpu:
         line["cpu_baseline"] = cpu_baseline(args, deck, stats)
     if rank == 0:
@@ -587,6 +620,8 @@ def main():
     ap.add_argument("--no-trace", action="store_true",
                     help="time without the in-graph kernel timing (no roofline block)")
     ap.add_argument("--no-cpu", action="store_true")
+    ap.add_argument("--no-variants", action="store_true",
+                    help="skip the CPPCG1F line of the headline run")
     args = ap.parse_args()
     if args.warmup < 3:
         ap.error("--warmup must be >= 3")

@@ -114,3 +114,21 @@ def test_listing1_dot_is_pw(ora):
     rng = np.random.default_rng(5)
     a, b = rng.standard_normal((7, 9)), rng.standard_normal((7, 9))
     assert ora.dot(a, b) == pytest.approx(float(np.sum(a * b)), rel=1e-13)
+
+
+@pytest.mark.parametrize("nx,ny,seed", [(17, 13, 0), (40, 31, 1), (1, 25, 2), (23, 1, 3)])
+def test_energy_form_of_zAz(ora, nx, ny, seed):
+    """z.(A z) = sum_c z_c^2 + sum_faces K_f (z_i - z_j)^2 (A = I + L, L the face-weighted graph
+    Laplacian of Listing 1): the identity the GPU's CPPCG1F last pass uses to form del = z.q
+    from z alone, each face counted once by its west / south cell (reading R23)."""
+    d = inputs.random_fields(nx, ny, seed, dt=0.4)
+    rx, ry = ora.mesh_r(d)
+    Kx, Ky = ora.face_coefficients(nx, ny, rx, ry, d.density)
+    z = np.random.default_rng(seed).standard_normal((ny, nx))
+    lhs = ora.dot(z, ora.apply_A(Kx, Ky, z))
+    # Kx[k, j] = face between cells j-1 and j (0 at the boundary columns), Ky[k, j] likewise
+    faces = np.sum(Kx[:, 1:nx] * (z[:, 1:] - z[:, :-1]) ** 2) + \
+        np.sum(Ky[1:ny, :] * (z[1:, :] - z[:-1, :]) ** 2)
+    rhs = np.sum(z * z) + faces
+    assert lhs == pytest.approx(rhs, rel=1e-13)
+    assert np.all(Kx[:, 0] == 0) and np.all(Kx[:, nx] == 0)  # reflective boundary (R3)
