@@ -104,6 +104,7 @@ def main():
     # traffic per launch for bench.py: average over the captured launches of each class
     key = {"k_cheb_tb<5, 1, 1, 0>": "tb_first", "k_cheb_tb<5, 0, 0, 1>": "tb_last",
            "k_cheb_tb<5, 1, 1, 0, 1>": "tb_first", "k_cheb_tb<5, 0, 0, 1, 1>": "tb_last",
+           "k_cheb_tb<5, 1, 1, 0, 1, 0, 0>": "tb_first", "k_cheb_tb<5, 0, 0, 1, 1, 0, 0>": "tb_last",
            "k_spmv<0>": "spmv", "k_spmv": "spmv"}
     tp = os.path.join(prof, "ncu_traffic.json")
     traffic = json.load(open(tp))
