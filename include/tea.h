@@ -228,7 +228,9 @@ tea_status tea_fetch(tea_ctx *ctx, double *u_host);
  * resume from a checkpoint written by tea_fetch. Host-synchronous.            */
 tea_status tea_set_u(tea_ctx *ctx, const double *u_host);
 
-/* Per-kernel-class device time accumulated since the last reset in profile mode:
+/* Per-kernel-class device time accumulated since the last reset in profile mode (eager
+ * launches bracketed by events: every HOST launch is counted, including the no-op launches
+ * issued after the solve finished -- tea_trace_read() counts only launches that did work):
  * ms[i], launches[i] and bytes[i] for i < TEA_K_COUNT (any may be NULL). bytes are
  * the ALGORITHMIC HBM bytes of those launches (fp64 streams x 8 B x owned cells, the
  * model of DESIGN.md §4; halos and redundant overlap compute excluded).

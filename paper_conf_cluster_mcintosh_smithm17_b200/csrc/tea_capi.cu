@@ -140,6 +140,10 @@ struct tea_ctx {
     cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
     Scalars *hS = nullptr;  // pinned host mirror (head only)
     ncclComm_t comm = nullptr;
+    // halos exchanged on the second stream use their own communicator (split from comm): an
+    // exchange there may run concurrently with an allreduce on the compute stream, and two
+    // concurrent NCCL operations must not share one communicator's connections
+    ncclComm_t xcomm = nullptr;
     std::string err;
     bool failed = false;
     long long launches = 0;
@@ -218,14 +222,19 @@ void wait_stream(tea_ctx *c) {
         if (q != cudaErrorNotReady) CK(q);
         ncclResult_t ar = ncclSuccess;
         NK(ncclCommGetAsyncError(c->comm, &ar));
+        if (ar == ncclSuccess && c->xcomm) NK(ncclCommGetAsyncError(c->xcomm, &ar));
         const double dt =
             std::chrono::duration<double>(std::chrono::steady_clock::now() - t0).count();
         if (ar != ncclSuccess && ar != ncclInProgress) {
+            if (c->xcomm) ncclCommAbort(c->xcomm);
+            c->xcomm = nullptr;
             ncclCommAbort(c->comm);
             c->comm = nullptr;
             fail(TEA_ERR_NCCL, "NCCL async error: %s", ncclGetErrorString(ar));
         }
         if (dt > timeout_s) {
+            if (c->xcomm) ncclCommAbort(c->xcomm);
+            c->xcomm = nullptr;
             ncclCommAbort(c->comm);
             c->comm = nullptr;
             fail(TEA_ERR_NCCL, "no completion after %.0f s (TEA_NCCL_TIMEOUT_S): a peer rank "
@@ -416,6 +425,7 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
             }
     if (remote) NK(ncclGroupStart());
     const int bpr = c->px * c->py / c->nranks;
+    const ncclComm_t hcomm = (xs && c->xcomm) ? c->xcomm : c->comm;
     for (auto &b : c->blocks) {
         const XPlan &x = b.xp[kind];
         for (int d = 0; d < kNDir; ++d) {
@@ -432,9 +442,9 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
                                    x.slen[d] * sizeof(double), cudaMemcpyDeviceToDevice,
                                    st));
             } else {
-                NK(ncclSend(b.sendbuf + x.soff[d], x.slen[d], ncclDouble, nrank, c->comm,
+                NK(ncclSend(b.sendbuf + x.soff[d], x.slen[d], ncclDouble, nrank, hcomm,
                             st));
-                NK(ncclRecv(b.recvbuf + x.roff[d], x.rlen[d], ncclDouble, nrank, c->comm,
+                NK(ncclRecv(b.recvbuf + x.roff[d], x.rlen[d], ncclDouble, nrank, hcomm,
                             st));
             }
         }
@@ -1603,6 +1613,7 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
             ncclUniqueId id;
             std::memcpy(&id, dist->nccl_id, sizeof id);
             NK(ncclCommInitRank(&c->comm, nranks, id, rank));
+            if (px * py > 1) NK(ncclCommSplit(c->comm, 0, rank, &c->xcomm, nullptr));
         }
 
         const int bpr = px * py / nranks;
@@ -1815,6 +1826,7 @@ tea_status tea_finalize(tea_ctx *ctx) {
     if (ctx->ev_join) cudaEventDestroy(ctx->ev_join);
     if (ctx->xstream) cudaStreamDestroy(ctx->xstream);
     if (ctx->hS) cudaFreeHost(ctx->hS);
+    if (ctx->xcomm) ncclCommDestroy(ctx->xcomm);
     if (ctx->comm) ncclCommDestroy(ctx->comm);
     if (ctx->stream) cudaStreamDestroy(ctx->stream);
     tb_slot_release(ctx->coef_slot);
