@@ -154,6 +154,21 @@ __device__ __forceinline__ void tm_st12(uint32_t a, double2 v0, double2 v1, doub
         "r"(d_hi(v2.x)), "r"(d_lo(v2.y)), "r"(d_hi(v2.y))
         : "memory");
 }
+#ifndef TEA_TB_STX2
+#define TEA_TB_STX2 1
+#endif
+// One double (an aligned register pair) into two TMEM columns: storing a row slot double by
+// double needs no operand marshalling (the x8 / x4 forms want 8 / 4 consecutive registers:
+// 16 register moves per row, profiles/r02c_ncu_summary.md)
+__device__ __forceinline__ void tm_st1(uint32_t a, double v) {
+    asm volatile("tcgen05.st.sync.aligned.32x32b.x2.b32 [%0], {%1, %2};" ::"r"(a), "r"(d_lo(v)),
+                 "r"(d_hi(v))
+                 : "memory");
+}
+__device__ __forceinline__ void tm_st2x(uint32_t a, double2 v) {
+    tm_st1(a, v.x);
+    tm_st1(a + 2u, v.y);
+}
 __device__ __forceinline__ void tm_st4(uint32_t a, double2 v) {
     asm volatile("tcgen05.st.sync.aligned.32x32b.x4.b32 [%0], {%1, %2, %3, %4};" ::"r"(a),
                  "r"(d_lo(v.x)), "r"(d_hi(v.x)), "r"(d_lo(v.y)), "r"(d_hi(v.y))
@@ -403,8 +418,12 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory");
     __syncthreads();
     asm volatile("tcgen05.fence::after_thread_sync;" ::: "memory");
-    const uint32_t tm = tm_base_sh + ((uint32_t)(((threadIdx.x >> 5) & 3) * 32) << 16) +
-                        (uint32_t)(((threadIdx.x >> 5) >> 2) * kTmCols);
+    // (broadcast from lane 0: a value the compiler knows is warp-uniform can stay in a
+    // uniform register, so the TMEM operations need no per-use register->uniform moves)
+    const uint32_t tm = __shfl_sync(0xffffffffu,
+                                    tm_base_sh + ((uint32_t)(((threadIdx.x >> 5) & 3) * 32) << 16) +
+                                        (uint32_t)(((threadIdx.x >> 5) >> 2) * kTmCols),
+                                    0);
     for (int d = 0; d < D; ++d) tm_st16(tm + 16u * d, z0, z0, z0, z0);  // zero ring
 
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -539,7 +558,13 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         // q+1): they wait in this thread's TMEM ring. The previous row's stores must land
         // before this row's loads read them back.
         tm_wait_st();
+#if TEA_TB_STX2
+        tm_st2x(tm + 16u * head, KX);
+        tm_st2x(tm + 16u * head + 4u, KY);
+        tm_st2x(tm + 16u * head + 8u, rk);
+#else
         tm_st12(tm + 16u * head, KX, KY, rk);
+#endif
         TmRow tmA;
         tm_ld12(tm + 16u * ((head + D - 1) % D), tmA);  // row k-1: level 1's operands
         tm_wait_ld(tmA);
@@ -553,7 +578,11 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         double2 s_d;
         s_d.x = 1.0 + (s_kx.x + s_kx.y) + (s_ky.x + KY.x);
         s_d.y = 1.0 + (s_kx.y + kxE) + (s_ky.y + KY.y);
+#if TEA_TB_STX2
+        tm_st2x(tm + 16u * ((head + D - 1) % D) + 12u, s_d);
+#else
         tm_st4(tm + 16u * ((head + D - 1) % D) + 12u, s_d);
+#endif
         const double2 z2row = z2prev;  // z_{i-2} of row k-1
         if (!FIRST) z2prev = Z2;
         W[0][0] = W[0][1];
@@ -586,7 +615,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                 // w = A p; r' = r - alpha w = r + alpha (sum_f K_f p_f - d p)
                 zn.x = fma(alpha, fma(kyn.x, xp.x, nb.x), rq.x);
                 zn.y = fma(alpha, fma(kyn.y, xp.y, nb.y), rq.y);
-                tm_st4(tm + 16u * ((head + D - 1) % D) + 8u, zn);  // row q's r is now r'
+                tm_st2x(tm + 16u * ((head + D - 1) % D) + 8u, zn);  // row q's r is now r'
                 if (rowout) st2m(rout + (orow - pitch), zn, oA, oB);
             } else if (POST && !POSTF && t == NL) {
                 // q = A z_s at row q (xc = z_s): z_s . q, and r . z_s, r . r of the same row
