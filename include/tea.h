@@ -74,7 +74,7 @@ typedef enum {
  * r -= alpha A p) and the first Chebyshev steps, the last pass the last steps and q = A z
  * with the three dot products -- 15 fp64 streams (TEA_CPPCG: 3 kernels, 18 streams; TEA_CPPCG1:
  * 4 kernels, 22). Same iterates as CPPCG in exact arithmetic; s + 2 matvecs per outer
- * iteration. 2D.                                                                     */
+ * iteration. 2D fused passes; 3D (and d < s + 1 blocks) by one kernel per step.       */
 typedef enum {
     TEA_CG = 0, TEA_CPPCG = 1, TEA_BJCG = 2, TEA_CG1 = 3, TEA_JACOBI = 4, TEA_CHEBY = 5,
     TEA_CPPCG1 = 6, TEA_CPPCG1F = 7

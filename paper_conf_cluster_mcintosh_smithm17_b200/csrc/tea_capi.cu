@@ -26,6 +26,12 @@
 
 using namespace tea;
 
+#ifndef TEA_CPPCG_UPD
+#define TEA_CPPCG_UPD 0  // 1: CPPCG fused passes do u += alpha p in the last pass instead of the
+                         // SpMV (measured slower: SpMV 165 -> 137 us but last pass 151 -> 199 us,
+                         // profiles/r02_upd_ab.txt)
+#endif
+
 namespace {
 
 constexpr int kNDir = 8;
@@ -697,6 +703,10 @@ struct ChainX {
     // passes); after the last pass z_s is exchanged at depth d + 1 while the chain's one
     // reduction [z.q, r.z, r.r] is in flight
     bool noexch = false, xz = false;
+    // CPPCG with the fused passes (faces from g): the last pass does u += alpha p with the
+    // direction the SpMV just wrote (field pnew); the SpMV then skips its lazy u update
+    bool upd = false;
+    int pnew = -1;
 };
 
 // Passes of a chain. CPPCG1F on one block (pre and post): an even number of passes >= 2, so
@@ -805,11 +815,12 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
                 ty *= 2;
             // algorithmic streams: reads, then writes
             int streams;
+            const bool upd = x.upd && last;
             if (pre)
                 streams = 4 + kstreams(c, b) + 3 + (last ? 1 : 2);  // z_s, p, r, u, g -> p, u, r', z..
             else
                 streams = (first ? (fu ? 2 : 1) : 3) + kstreams(c, b) + (fu ? 1 : 0) +
-                          (last ? 1 : 2);  // writes: r', z_last(, z_{last-1})
+                          (last ? 1 : 2) + (upd ? 3 : 0);  // writes: r', z_last(, z_{last-1}); p, u -> u
             const int kid = last ? TEA_K_TB_LAST : (first ? TEA_K_TB_FIRST : TEA_K_TB_MID);
             TbArgs f;
             f.rin = b.f[first && (fu || pre) ? rin : r];
@@ -826,9 +837,13 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
                 f.pout = b.f[x.pout];
                 f.uio = b.f[F_U];
             }
+            if (upd) {
+                f.pin = b.f[x.pnew];
+                f.uio = b.f[F_U];
+            }
             K(c, kid, sbytes(b, streams), [&] {
                 launch_cheb_tb(kargs(c, b, last && sets_cond), R, D, M, ty, jlim, step0, first,
-                               fu, last, restart, pre, post, f, c->stream);
+                               fu, last, restart, pre, post, upd, f, c->stream);
             });
           }
         }
@@ -900,12 +915,15 @@ int zs_field1f(tea_ctx *c, int s) {
 void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
     const bool fused = single_block(c);
     const int zs = zs_field(c, s);
+    // with the fused passes and faces from g the last pass updates u (the SpMV's lazy update
+    // moved where HBM bandwidth is idle: SpMV 7 -> 5 streams, last pass 5 -> 8)
+    const bool upd = TEA_CPPCG_UPD && use_tb(c, s) && c->opts.kform >= 0;
     for (auto &b : c->blocks) {
         Region R = b.owned();
         Launch L = plan_spmv(c, b, R);
-        K(c, TEA_K_SPMV, sbytes(b, 6 + kstreams(c, b)), [&] {
+        K(c, TEA_K_SPMV, sbytes(b, (upd ? 4 : 6) + kstreams(c, b)), [&] {
             launch_spmv(kargs(c, b), L, R, b.f[zs], b.f[F_P0 + par], b.f[F_P1 - par],
-                        b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream);
+                        b.f[F_W], b.f[F_U], b.f[F_KX], b.f[F_KY], c->stream, !upd);
         });
     }
     if (!fused && use_tb(c, s)) {
@@ -914,11 +932,18 @@ void body_pcg(tea_ctx *c, int s, int par, bool sets_cond) {
         // streams), and the exchange overlaps the p.w reduction
         ChainX x;
         x.xw = true;
+        x.upd = upd;
+        x.pnew = F_P1 - par;
         cheb_chain_tb(c, s, false, true, F_R0 + par, F_R1 - par, sets_cond, true, x);
         return;
     }
     reduce(c, 0, 1);
-    if (fused) {
+    if (fused && use_tb(c, s)) {
+        ChainX x;
+        x.upd = upd;
+        x.pnew = F_P1 - par;
+        cheb_chain_tb(c, s, false, true, F_R0 + par, F_R1 - par, sets_cond, true, x);
+    } else if (fused) {
         chain(c, s, false, true, F_R0 + par, F_R1 - par, sets_cond);
     } else {
         for (auto &b : c->blocks) {

@@ -344,7 +344,11 @@ constexpr int kTmCols = 128;  // TMEM columns per 4 warps: 8 slots x 16 per warp
 // one more stencil level q = A z_s whose z_s . q joins r.z and r.r in ONE grid reduction.
 // alpha and beta come from the previous reduction (Chronopoulos & Gear). Every level loses a
 // column per side and lags a row: NL = M + PRE + POST <= 6 levels.
-template <int M, bool FIRST, bool FUSE, bool LAST, bool KG, bool PRE, bool POST>
+// UPD (CPPCG with faces from g, last pass): u += alpha p at the input rows, alpha = this
+// iteration's (alpha_prev, set by the first pass) and p the direction the SpMV just wrote --
+// the update the SpMV otherwise applies lazily, moved to the compute-bound last pass whose HBM
+// bandwidth is idle (SpMV 7 -> 5 streams, this pass 5 -> 8).
+template <int M, bool FIRST, bool FUSE, bool LAST, bool KG, bool PRE, bool POST, bool UPD = false>
 __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     k_cheb_tb(const double *__restrict__ rin, const double *__restrict__ win,
               double *__restrict__ rout, const double *__restrict__ zin1,
@@ -365,6 +369,10 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     static_assert(NL <= 6, "the TMEM ring holds NL+2 rows");
     static_assert(!PRE || (FIRST && !FUSE && KG), "PRE: first pass, g faces, no FUSE update");
     static_assert(!POST || LAST, "POST: last pass");
+    static_assert(!UPD || (LAST && KG && !PRE && !POST), "UPD: last pass, g faces");
+    // staged streams per row: X, W / z_{i-2}, r, Kx (g), Ky -- UPD adds p and u
+    constexpr int NS = (UPD && !FIRST) ? 6 : kTbNS;
+    constexpr int PSL = FIRST ? 2 : 4, USL = FIRST ? 4 : 5;  // UPD's p / u slots
     static_assert(kTbW <= 4 || kTbW % 4 == 0, "warp quarters");
     extern __shared__ double2 tb_smem[];
     const double(*coef)[kMaxS] = c_tb_coef[a.coef_slot];
@@ -401,6 +409,8 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         alpha = cf.alpha;
         beta = cf.beta;
     }
+    // UPD: this iteration's alpha (FUSE computed it here; otherwise the first pass recorded it)
+    const double ualpha = UPD ? (FUSE ? alpha : S->alpha_prev) : 0.0;
     trace_begin(a);
     const double2 z0 = make_double2(0.0, 0.0);
     // One warp allocates the CTA's TMEM columns; warp w then owns lanes 32(w%4).. and a
@@ -461,10 +471,11 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     // warp. With one register-prefetched row the pass stalled on the load of the next row
     // (ncu: 41% of stall samples on its first use; profiles/r01g_tmem_cpa.txt).
     constexpr int P = FIRST ? kTbCpa : kTbCpaL, NSL = P + 1;
-    double2(*cpa)[kTbNS][kTbT] = reinterpret_cast<double2(*)[kTbNS][kTbT]>(tb_smem);
+    static_assert(NS * NSL <= kTbNS * (kTbCpa + 1), "staging fits the dynamic shared memory");
+    double2(*cpa)[NS][kTbT] = reinterpret_cast<double2(*)[NS][kTbT]>(tb_smem);
     for (int sl = 0; sl < NSL; ++sl)
 #pragma unroll
-        for (int q = 0; q < kTbNS; ++q) cpa[sl][q][threadIdx.x] = z0;
+        for (int q = 0; q < NS; ++q) cpa[sl][q][threadIdx.x] = z0;
     auto issue = [&](int o, int sl) {
         if (ld_ok) {
             if (PRE) {  // z_s, p_old, r, g, u
@@ -482,6 +493,10 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             }
             cp16(&cpa[sl][3][threadIdx.x], Kx + o);
             if (!KG) cp16(&cpa[sl][4][threadIdx.x], Ky + o);
+            if (UPD) {
+                cp16(&cpa[sl][PSL][threadIdx.x], pin + o);
+                cp16(&cpa[sl][USL][threadIdx.x], uio + o);
+            }
         }
         cp_commit();  // one group per row, empty or not, so wait_group counts rows
     };
@@ -519,6 +534,10 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             KY = cpa[cs][4][threadIdx.x];
         }
         double2 Wv = z0, Z2 = z0, RR = z0, PO = z0, UU = z0;
+        if (UPD) {
+            PO = cpa[cs][PSL][threadIdx.x];
+            UU = cpa[cs][USL][threadIdx.x];
+        }
         if (PRE) {
             PO = cpa[cs][1][threadIdx.x];
             RR = cpa[cs][2][threadIdx.x];
@@ -554,6 +573,8 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         } else {
             rk = RR;
         }
+        if (UPD && k >= kt0 && k < kt1 && k >= Dd.k0 && k < Dd.k1)  // owned cells only
+            st2m(uio + orow, make_double2(UU.x + ualpha * PO.x, UU.y + ualpha * PO.y), dA, dB);
         // level t works on row q = k - t and needs that row's Kx, Ky, r (and Ky of row
         // q+1): they wait in this thread's TMEM ring. The previous row's stores must land
         // before this row's loads read them back.
@@ -736,6 +757,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             S->red_rr = tot[1];
             if (POST) S->red_pw = tot[2];
             if (FUSE) S->alpha_prev = alpha;
+            if (UPD) S->alpha_prev = 0.0;  // u is current: nothing pending for the SpMV
             if (!restart) {
                 S->it += 1;
                 S->outer += 1;
@@ -762,7 +784,7 @@ int tb_out_cols(int NL) {
     return kTbW * ow;
 }
 
-template <int M, bool FIRST, bool FUSE, bool LAST, bool KG, bool PRE, bool POST>
+template <int M, bool FIRST, bool FUSE, bool LAST, bool KG, bool PRE, bool POST, bool UPD = false>
 static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty, int jlim,
                       int step0, bool restart, const TbArgs &f, cudaStream_t st) {
     constexpr int NL = M + (PRE ? 1 : 0) + ((POST && (M + (PRE ? 1 : 0)) % 2 == 0) ? 1 : 0);
@@ -774,13 +796,13 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
     static std::atomic<unsigned long long> attr{0ull};  // per instantiation: device bit mask
     const unsigned long long bit = 1ull << tea_device();
     if (!(attr.load() & bit)) {
-        cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST, KG, PRE, POST>,
+        cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST, KG, PRE, POST, UPD>,
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST, KG, PRE, POST>,
+        cudaFuncSetAttribute(k_cheb_tb<M, FIRST, FUSE, LAST, KG, PRE, POST, UPD>,
                              cudaFuncAttributePreferredSharedMemoryCarveout, 100);
         attr.fetch_or(bit);
     }
-    k_cheb_tb<M, FIRST, FUSE, LAST, KG, PRE, POST><<<grid, kTbT, smem, st>>>(
+    k_cheb_tb<M, FIRST, FUSE, LAST, KG, PRE, POST, UPD><<<grid, kTbT, smem, st>>>(
         f.rin, f.win, f.rout, f.zin1, f.zin2, f.zoutA, f.zoutB, KG ? a.g : f.kx, f.ky, f.pin,
         f.pout, f.uio, a, R, Dd, ty, jlim, step0, restart ? 1 : 0);
 }
@@ -788,7 +810,16 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
 template <int M>
 static void tb_dispatch(const KArgs &a, const Region &R, const Region &Dd, int ty, int jlim,
                         int step0, bool first, bool fuse, bool last, bool restart, bool pre,
-                        bool post, const TbArgs &f, cudaStream_t st) {
+                        bool post, bool upd, const TbArgs &f, cudaStream_t st) {
+    if (upd && last && a.g && !pre && !post) {  // CPPCG: u += alpha p in the last pass
+        if (!first)
+            tb_launch<M, false, false, true, true, false, false, true>(a, R, Dd, ty, jlim, step0, restart, f, st);
+        else if (fuse)
+            tb_launch<M, true, true, true, true, false, false, true>(a, R, Dd, ty, jlim, step0, restart, f, st);
+        else
+            tb_launch<M, true, false, true, true, false, false, true>(a, R, Dd, ty, jlim, step0, restart, f, st);
+        return;
+    }
 #define TB(F, U, L)                                                                       \
     do {                                                                                  \
         if (a.g)                                                                          \
@@ -910,13 +941,13 @@ int tb_ctas(int NL, int width, int height, int ty) {
 
 void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, int ty, int jlim,
                     int step0, bool first, bool fuse, bool last, bool restart, bool pre,
-                    bool post, const TbArgs &f, cudaStream_t st) {
+                    bool post, bool upd, const TbArgs &f, cudaStream_t st) {
     switch (M) {
-        case 1: tb_dispatch<1>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, f, st); break;
-        case 2: tb_dispatch<2>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, f, st); break;
-        case 3: tb_dispatch<3>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, f, st); break;
-        case 4: tb_dispatch<4>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, f, st); break;
-        default: tb_dispatch<5>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, f, st); break;
+        case 1: tb_dispatch<1>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, upd, f, st); break;
+        case 2: tb_dispatch<2>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, upd, f, st); break;
+        case 3: tb_dispatch<3>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, upd, f, st); break;
+        case 4: tb_dispatch<4>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, upd, f, st); break;
+        default: tb_dispatch<5>(a, R, Dd, ty, jlim, step0, first, fuse, last, restart, pre, post, upd, f, st); break;
     }
 }
 

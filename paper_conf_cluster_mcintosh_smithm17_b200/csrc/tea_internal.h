@@ -195,9 +195,10 @@ void launch_init_fields3(const KArgs &a, const double *rho, const double *en, do
 void launch_residual(const KArgs &a, const Launch &L, const Region &R, const double *u,
                      const double *kx, const double *ky, double *u0, double *r,
                      cudaStream_t st);
+// lazy_u = false: no u += alpha_prev p_old (2D; the last fused pass does the update)
 void launch_spmv(const KArgs &a, const Launch &L, const Region &R, const double *src,
                  const double *pin, double *pout, double *w, double *u, const double *kx,
-                 const double *ky, cudaStream_t st);
+                 const double *ky, cudaStream_t st, bool lazy_u = true);
 void launch_update(const KArgs &a, const Launch &L, const Region &R, const double *w,
                    double *r, cudaStream_t st);
 void launch_update_nodot(const KArgs &a, const Launch &L, const Region &R, const double *w,
@@ -275,10 +276,11 @@ int tb_slot_acquire();  // -1: none free (the context then uses per-step kernels
 void tb_slot_release(int slot);
 cudaError_t tb_coef_upload(int slot, const Scalars *S, cudaStream_t st);
 // M Chebyshev steps in one pass; pre: the CPPCG1F outer update first (first pass, g faces),
-// post: q = A z_s and z_s.q after the last step (last pass, g faces)
+// post: q = A z_s and z_s.q after the last step (last pass, g faces); upd: u += alpha p in
+// the last pass (CPPCG, g faces; the SpMV then runs without its lazy u update)
 void launch_cheb_tb(const KArgs &a, const Region &R, const Region &Dd, int M, int ty, int jlim,
                     int step0, bool first, bool fuse, bool last, bool restart, bool pre,
-                    bool post, const TbArgs &f, cudaStream_t st);
+                    bool post, bool upd, const TbArgs &f, cudaStream_t st);
 
 // Persistent single-launch CG / CPPCG solve of one 2D block (tea_kernels.cu, k_persist):
 // phases separated by grid-wide barriers of a cooperative launch.

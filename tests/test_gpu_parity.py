@@ -519,7 +519,7 @@ def deck3_of(kind, nx, ny, nz, seed=0, dt=0.004):
     return inputs.random_fields3(nx, ny, nz, seed, dt=dt)
 
 
-@pytest.mark.parametrize("method", [0, 1, 3, 4, 5, 6])
+@pytest.mark.parametrize("method", [0, 1, 3, 4, 5, 6, 7])
 @pytest.mark.parametrize("kind,nx,ny,nz", [("pipe", 40, 36, 28), ("random", 33, 17, 9),
                                            ("random", 70, 5, 2)])
 def test_3d_converged(tea, ora, method, kind, nx, ny, nz):
@@ -532,7 +532,7 @@ def test_3d_converged(tea, ora, method, kind, nx, ny, nz):
     assert field_err(u_g, u_o, kind) <= 1e-10
 
 
-@pytest.mark.parametrize("method,k", [(0, 3), (1, 33), (3, 4), (4, 5), (5, 35), (6, 33)])
+@pytest.mark.parametrize("method,k", [(0, 3), (1, 33), (3, 4), (4, 5), (5, 35), (6, 33), (7, 33)])
 def test_3d_fixed_iterations(tea, ora, method, k):
     deck = deck3_of("random", 45, 23, 11, seed=2, dt=0.04)
     kw = dict(method=method, eps=0.0, max_iters=k, inner_steps=5)

@@ -22,12 +22,17 @@ def main():
         (inputs.random_fields(300, 41, 5), None, dict(persist=1, loop_mode=0, tile_rows=1)),
         # fused passes across blocks with the halo exchange overlapped (second stream)
         (inputs.random_fields(90, 60, 4), dict(px=2, py=2, halo_depth=11, nranks=1),
-         dict(tb_steps=5, overlap=1, _s=10, _methods=(1, 6))),
+         dict(tb_steps=5, overlap=1, _s=10, _methods=(1, 6, 7))),
+        # single-reduction CPPCG, fused form: one block (pre / post passes, s = 10 and 4)
+        (inputs.crooked_pipe(96, 70), None, dict(tb_steps=5, _s=10, _methods=(7,))),
+        (inputs.random_fields(70, 50, 6), None, dict(tb_steps=5, _s=4, _methods=(7,))),
+        (inputs.random_fields(70, 50, 6), dict(px=2, py=1, halo_depth=2, nranks=1),
+         dict(_s=6, _methods=(7,))),
     ]
     for deck, dist, kw in cases:
         kw = dict(kw)
         s = kw.pop("_s", 4)
-        methods = kw.pop("_methods", (0, 1, 2, 3, 4, 5, 6))
+        methods = kw.pop("_methods", (0, 1, 2, 3, 4, 5, 6, 7))
         for method in methods:
             if getattr(deck, "nz", 1) > 1 and method == 2:
                 continue
