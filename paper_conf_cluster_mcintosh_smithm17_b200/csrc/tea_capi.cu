@@ -468,6 +468,27 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
     (void)nb;
 }
 
+// The reduction that ends an iteration and the depth-1 halo exchange of the field the next
+// stencil pass reads (CG: r with [r.r]; block Jacobi: z with [r.z, r.r]; Jacobi / Chebyshev:
+// u with [r.r]) depend on the same kernel and not on each other: with the overlap on (auto
+// across processes) the exchange runs on the second stream (its own communicator) while the
+// allreduce is in flight on the compute stream ("the r halo exchange is issued
+// together with the rr allreduce"); joined before the next iteration.
+void reduce_exchange(tea_ctx *c, int first, int n, int kind, const std::vector<int> &fields) {
+    const bool want = c->opts.overlap > 0 || (c->opts.overlap == 0 && c->nranks > 1);
+    if (c->px * c->py > 1 && c->xstream && want && !c->profiling) {
+        CK(cudaEventRecord(c->ev_fork, c->stream));
+        CK(cudaStreamWaitEvent(c->xstream, c->ev_fork, 0));
+        exchange(c, kind, fields, c->xstream);
+        CK(cudaEventRecord(c->ev_join, c->xstream));
+        reduce(c, first, n);
+        CK(cudaStreamWaitEvent(c->stream, c->ev_join, 0));
+        return;
+    }
+    reduce(c, first, n);
+    exchange(c, kind, fields);
+}
+
 // Boxes of owned cells sent to direction d, and halo cells received from it.
 void send_box(const BlockLayout &L, int d, int dep, int *j0, int *j1, int *k0, int *k1) {
     *j0 = 0;
@@ -618,8 +639,7 @@ void body_cg(tea_ctx *c, int par, bool last_sets_cond) {
             launch_update(kargs(c, b, last_sets_cond), L, R, b.f[F_W], b.f[F_R0], c->stream);
         });
     }
-    reduce(c, 1, 2);
-    exchange(c, X_R1, {F_R0});
+    reduce_exchange(c, 1, 2, X_R1, {F_R0});
 }
 
 // Chebyshev chain z = B(A) r, one kernel per step (blocks with neighbours; or
@@ -975,8 +995,7 @@ void body_bj(tea_ctx *c, int par, bool sets_cond) {
                       b.f[F_KY], b.f[F_BJC], b.f[F_BJD], c->stream);
         });
     }
-    reduce(c, 1, 2);
-    exchange(c, X_Z1, {F_Z0});
+    reduce_exchange(c, 1, 2, X_Z1, {F_Z0});
 }
 
 // Single-reduction CG iteration (Chronopoulos-Gear): one fused kernel on a
@@ -1107,8 +1126,7 @@ void body_stat(tea_ctx *c, bool cheb, int par, bool sets_cond) {
                         b.f[F_KX], b.f[F_KY], c->stream);
         });
     }
-    reduce(c, 2, 1);
-    exchange(c, X_U1, {out});
+    reduce_exchange(c, 2, 1, X_U1, {out});
 }
 
 void read_state(tea_ctx *c) {

@@ -838,3 +838,19 @@ def test_cppcg1f_blocks_overlap_bitwise(tea, ora, nx, ny, px, py, d, loop_mode):
     u_o, st_o, _ = ora.run(deck, steps=1, method=7, eps=0.0, max_iters=35, inner_steps=s)
     assert iter_err(u_a, u_o, "random") <= 1e-12
     assert st_a[0]["rnorm"] == pytest.approx(st_o[0]["rnorm"], rel=1e-9)
+
+
+@pytest.mark.parametrize("method", [0, 2, 4, 5])
+@pytest.mark.parametrize("px,py", [(2, 2), (3, 1)])
+@pytest.mark.parametrize("loop_mode", [0, 2])
+def test_reduce_exchange_overlap_bitwise(tea, method, px, py, loop_mode):
+    """CG / block-Jacobi / Jacobi / Chebyshev across blocks: the depth-1 halo exchange issued
+    on the second stream together with the iteration's reduction (overlap on) gives bitwise
+    the same solve as exchange-after-reduction (overlap off)."""
+    deck = deck_of("random", 130, 97, seed=11, dt=0.04)
+    kw = dict(method=method, eps=1e-12, max_iters=3000, presteps=10, loop_mode=loop_mode,
+              dist=dict(px=px, py=py, halo_depth=1, nranks=1))
+    u_a, st_a = gpu_run(tea, deck, overlap=1, **kw)
+    u_b, st_b = gpu_run(tea, deck, overlap=-1, **kw)
+    assert st_a[0]["iterations"] == st_b[0]["iterations"]
+    assert np.array_equal(u_a, u_b)
