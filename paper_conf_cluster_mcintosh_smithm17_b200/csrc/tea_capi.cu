@@ -366,7 +366,12 @@ Launch plan_spmv(tea_ctx *c, const BlockCtx &b, const Region &R) {
         const int gz = std::max(1, 592 / std::max(cols, 1));
         return checked(b, plan_stencil3(R, b.L.nz, std::max(4, (b.L.nz + gz - 1) / gz)));
     }
-    if (b.L.nz > 1 || c->opts.tile_rows > 0 || c->ty_override > 0 || L.ty < 32) return L;
+    if (b.L.nz > 1 || c->opts.tile_rows > 0 || c->ty_override > 0) return L;
+    // blocks >= 2M cells get whole waves too (2048 x 1024, the 8-GPU 4096^2 block: the
+    // default 8-row tiles were 1.4 waves of 740 slots); smaller ones keep plan_stencil's
+    // latency-tuned short tiles (1024^2: 8 rows, the measured optimum)
+    const double cells = (double)(R.j1 - R.j0) * (R.k1 - R.k0);
+    if (L.ty < 32 && cells < 2.0e6) return L;
     const int ty = spmv_wave_rows(R.j1 - L.jstart, R.k1 - R.k0);
     // one reduction partial per CTA must fit the block's scratch (fewer CTAs: always true)
     return checked(b, plan_stencil(R, ty, 0));
