@@ -58,7 +58,7 @@ struct BlockLayout {
     int nz;          // planes (1: 2D)
     long long ps;    // plane stride (doubles), rows * pitch
     int H, X0, pitch, rows, planes;
-    size_t field_bytes, scalars_off, partials_off, partials_cap, boxes_off, halo_off,
+    size_t field_bytes, scalars_off, partials_off, partials_cap, boxes_off, xdesc_off, halo_off,
         halo_cap, total;
     bool has_nbr;
 };
@@ -101,6 +101,9 @@ BlockLayout layout_block(const tea_mesh &m, int px, int py, int d, int b) {
     L.has_nbr = (px * py > 1);
     L.boxes_off = off;
     off += L.has_nbr ? 16384 : 0;
+    // direct-exchange descriptors of every block of the process (used in block 0's copy)
+    L.xdesc_off = off;
+    off += L.has_nbr ? round_up((size_t)X_COUNT * px * py * 16 * sizeof(XCopy), 256) : 0;
     L.halo_off = off;
     // per field and depth d: two faces in x, two in y, four corners
     size_t per_field = 2 * (size_t)d * (L.bx + L.by) + 4 * (size_t)d * d;
@@ -166,6 +169,9 @@ struct tea_ctx {
     std::map<long long, int> graph_kernels;
     // capture state
     cudaGraphConditionalHandle cond = 0;
+    // direct in-process halo exchange (all blocks local): descriptors per exchange kind
+    XCopy *xdesc[16] = {};
+    int nxdesc[16] = {};
     // in-graph kernel timing (tea_opts.trace): slot i times launches of (kid, bytes)
     std::vector<std::pair<int, double>> tslots;
     int cur_tslot = -1;
@@ -426,6 +432,21 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
         });
     }
     // transport
+    bool remote0 = false;
+    for (auto &b : c->blocks)
+        for (int d = 0; d < kNDir; ++d)
+            if (b.nbr[d] >= 0 && b.nbr[d] / (c->px * c->py / c->nranks) != c->rank) remote0 = true;
+    if (!remote0 && c->nxdesc[kind] > 0) {
+        // every neighbour is in this process: one direct-copy launch, no pack / copy / unpack
+        XFields F{};
+        for (size_t i = 0; i < c->blocks.size() && i < (size_t)kXMaxBlocks; ++i) {
+            for (int j = 0; j < nf && j < 2; ++j) F.f[i][j] = c->blocks[i].f[fids_per_block_field[j]];
+            F.pitch[i] = c->blocks[i].L.pitch;
+        }
+        K(c, TEA_K_PACK, 0.0, [&] { launch_xcopy(c->xdesc[kind], c->nxdesc[kind], F, st); });
+        return;
+    }
+    // transport
     bool remote = false;
     for (auto &b : c->blocks)
         for (int d = 0; d < kNDir; ++d)
@@ -560,6 +581,44 @@ void build_xplans(tea_ctx *c, BlockCtx &b, int *d_boxes_base) {
                            c->stream));
         dptr += 16 * 5 * 2;
         CK(cudaStreamSynchronize(c->stream));
+    }
+}
+
+// Descriptors of the direct in-process exchange (k_xcopy): for every block, neighbour direction
+// and field of each exchange kind, the send box of the block and the matching receive box of
+// the neighbour (same shapes as the packed path's).
+void build_xcopy(tea_ctx *c) {
+    struct K2 {
+        int nf, dep;
+        bool corners;
+    } kinds[X_COUNT] = {{1, 1, false}, {1, c->d, c->d > 1}, {2, c->d, c->d > 1},
+                        {1, 1, false}, {1, 1, false}, {1, c->d + 1, true}};
+    const BlockCtx &b0 = c->blocks[0];
+    XCopy *base = (XCopy *)((char *)b0.S - b0.L.scalars_off + b0.L.xdesc_off);
+    const size_t per_kind = (size_t)c->px * c->py * 16;
+    for (int kd = 0; kd < X_COUNT; ++kd) {
+        std::vector<XCopy> v;
+        for (size_t i = 0; i < c->blocks.size(); ++i) {
+            const BlockCtx &b = c->blocks[i];
+            for (int d = 0; d < kNDir; ++d) {
+                if (b.nbr[d] < 0 || (d >= 4 && !kinds[kd].corners)) continue;
+                const int nl = b.nbr[d] - c->rank * (int)c->blocks.size();
+                const BlockCtx &nb = c->blocks[nl];
+                int sj0, sj1, sk0, sk1, dj0, dj1, dk0, dk1;
+                send_box(b.L, d, kinds[kd].dep, &sj0, &sj1, &sk0, &sk1);
+                recv_box(nb.L, kOpp[d], kinds[kd].dep, &dj0, &dj1, &dk0, &dk1);
+                if (sj1 - sj0 != dj1 - dj0 || sk1 - sk0 != dk1 - dk0)
+                    fail(TEA_ERR_STATE, "direct exchange box mismatch");
+                for (int f = 0; f < kinds[kd].nf; ++f)
+                    v.push_back(XCopy{(int)i, nl, f, sj0, sk0, dj0, dk0, sj1 - sj0, sk1 - sk0});
+            }
+        }
+        if (v.size() > per_kind) fail(TEA_ERR_STATE, "direct exchange table too small");
+        c->xdesc[kd] = base + kd * per_kind;
+        c->nxdesc[kd] = (int)v.size();
+        if (!v.empty())
+            CK(cudaMemcpyAsync(c->xdesc[kd], v.data(), v.size() * sizeof(XCopy),
+                               cudaMemcpyHostToDevice, c->stream));
     }
 }
 
@@ -1741,6 +1800,7 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
             CK(cudaMemsetAsync(ws + F_Z0 * L.field_bytes, 0, L.field_bytes, c->stream));
             ws += L.total;
         }
+        if (nranks == 1 && px * py > 1 && bpr <= kXMaxBlocks) build_xcopy(c.get());
         CK(cudaStreamSynchronize(c->stream));
         c->coef_slot = tb_slot_acquire();
         *out = c.release();

@@ -217,6 +217,17 @@ void launch_scalars(const KArgs &a, int mode, double eps, int it_limit, int max_
 void launch_combine(Scalars *const *S_dev_list, int nblocks, int nvals, int first_slot,
                     cudaStream_t st);
 void launch_mask_done(Scalars *S, int first, int nvals, bool zero, cudaStream_t st);
+// direct in-process halo exchange (k_xcopy): box e copies src block's field fld at
+// (sj0.., sk0..) into dst block's field fld at (dj0.., dk0..), w x h cells
+struct XCopy {
+    int src, dst, fld, sj0, sk0, dj0, dk0, w, h;
+};
+constexpr int kXMaxBlocks = 64;
+struct XFields {
+    double *f[kXMaxBlocks][2];
+    int pitch[kXMaxBlocks];
+};
+void launch_xcopy(const XCopy *desc, int n, const XFields &F, cudaStream_t st);
 void launch_pack(const double *const *fields, int nf, int pitch, const int *boxes,
                  int nbox, double *buf, cudaStream_t st);
 void launch_unpack(double *const *fields, int nf, int pitch, const int *boxes, int nbox,
