@@ -102,17 +102,23 @@ def main():
     import bench
     shash = bench.source_hash()
     # traffic per launch for bench.py: average over the captured launches of each class
-    key = {"k_cheb_tb<5, 1, 1, 0>": "tb_first", "k_cheb_tb<5, 0, 0, 1>": "tb_last",
-           "k_cheb_tb<5, 1, 1, 0, 1>": "tb_first", "k_cheb_tb<5, 0, 0, 1, 1>": "tb_last",
-           "k_cheb_tb<5, 1, 1, 0, 1, 0, 0>": "tb_first", "k_cheb_tb<5, 0, 0, 1, 1, 0, 0>": "tb_last",
-           "k_spmv<0>": "spmv", "k_spmv": "spmv"}
+    # kernel class of a full-set entry: template-argument prefixes of the headline's kernels
+    # (the argument lists grew over the rounds: <M, FIRST, FUSE, LAST[, KG[, PRE, POST[, UPD]]]>)
+    prefixes = [("k_cheb_tb<5, 1, 1, 0", "tb_first"), ("k_cheb_tb<5, 0, 0, 1", "tb_last"),
+                ("k_spmv<0", "spmv"), ("k_spmv", "spmv")]
+
+    def cls_of(name):
+        for pre, c in prefixes:
+            if name.startswith(pre):
+                return c
+        return None
     tp = os.path.join(prof, "ncu_traffic.json")
     traffic = json.load(open(tp))
     per = defaultdict(list)
     for k in full:
         name = k["kernel"].replace("void ", "")
-        if name in key:
-            per[key[name]].append((k["dram_read_bytes"] + k["dram_write_bytes"], k["kernel"]))
+        if cls_of(name):
+            per[cls_of(name)].append((k["dram_read_bytes"] + k["dram_write_bytes"], k["kernel"]))
     for cls, v in per.items():
         ent = traffic.setdefault(f"{cls}@{n}", {})
         ent["dram_bytes_per_launch"] = int(sum(x for x, _ in v) / len(v))
@@ -121,7 +127,7 @@ def main():
         ent["kernel"] = v[0][1]
         ent["round"] = tag[1:] if tag.startswith("r") else tag
         ent["source_hash"] = shash
-        ent["capture"] = f"ncu --set full, gpurun_out/prof_{tag}, summary profiles/{tag}_ncu_summary.md"
+        ent["capture"] = f"ncu --set full, gpurun_out/prof_{tag}" + (f", summary {sys.argv[3]}" if len(sys.argv) > 3 else "")
     json.dump(traffic, open(tp, "w"), indent=1)
     tot = sum(a[1] for a in agg.values()) or 1.0
     totw = sum(a[1] for a in aggw.values()) or 1.0
