@@ -105,3 +105,34 @@ def test_16384_every_cell(tea, ora):
         assert r.stats["rnorm"] == pytest.approx(st_o["rnorm"], rel=1e-9)
         assert r.stats["eig_max"] == pytest.approx(st_o["eig_max"], rel=1e-9)
     assert e1 <= TOL and e8 <= TOL and e18 <= TOL
+
+
+_conv = {}
+
+
+@pytest.mark.parametrize("method", [0, 1, 7])
+def test_1024_converged_every_cell(tea, ora, method):
+    """configs[1]: 1024^2, CG vs CPPCG (and the single-reduction CPPCG), converged to
+    eps = 1e-12 in the bench's configuration, against the oracle run live: every cell within
+    the north_star's 1e-10, iteration counts within +-2; CG and CPPCG within the R22 bound."""
+    from paper_conf_cluster_mcintosh_smithm17_b200 import inputs
+    deck = inputs.crooked_pipe(1024)
+    u_o, st_o, s_o = ora.run(deck, steps=1, method=method, eps=1e-12, max_iters=20000,
+                             inner_steps=10)
+    u_g, r = gpu_run(tea, deck, None, method=method, eps=1e-12, max_iters=20000, inner_steps=10)
+    err = pointwise(u_g, u_o)
+    print(f"\n1024^2 method={method}: iterations gpu {r.stats['iterations']} oracle "
+          f"{st_o[0]['iterations']}, max pointwise rel err {err:.3e}")
+    assert s_o[0] == 0 and r.status == 0
+    assert abs(r.stats["iterations"] - st_o[0]["iterations"]) <= 2
+    assert err <= TOL
+    _conv[method] = u_g
+    if 0 in _conv and method != 0:
+        # CG and CPPCG stop at the same relative residual, not at the same error: their fields
+        # differ by ~kappa eps (1e-9 here), bounded per cell by the two true residual norms
+        # (lambda_min(A) = 1, reading R22)
+        rx, ry = ora.mesh_r(deck)
+        Kx, Ky = ora.face_coefficients(1024, 1024, rx, ry, deck.density)
+        u0 = deck.density * deck.energy
+        bound = sum(float(np.linalg.norm(u0 - ora.apply_A(Kx, Ky, u))) for u in (u_g, _conv[0]))
+        assert float(np.max(np.abs(u_g - _conv[0]))) <= bound
