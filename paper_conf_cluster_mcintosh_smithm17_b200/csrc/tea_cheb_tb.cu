@@ -273,20 +273,13 @@ __device__ bool grid_arrive2(unsigned *ticket) {
 
 }  // namespace
 
-#ifndef TEA_TB_UNROLL
-#define TEA_TB_UNROLL 3
-#endif
-#ifndef TEA_TB_UNROLL_L
-#define TEA_TB_UNROLL_L 3
-#endif
 #ifndef TEA_TB_CPA_L
 #define TEA_TB_CPA_L 2
 #endif
-// Row-loop unroll and cp.async depth of the first pass (carries r, w and the update) and of
-// the later passes, measured separately (profiles/r01g_tmem_cpa.txt): unrolling by the
-// window period 3 turns the W[t][*] rotation into register renaming instead of ~50 moves per
-// row; with 3 CTAs per SM requested (TEA_TB_MINB) the first pass still fits 152 registers.
-constexpr int kTbUnroll = TEA_TB_UNROLL, kTbUnrollL = TEA_TB_UNROLL_L;
+// cp.async depth of the first pass (carries r, w and the update) and of the later passes,
+// measured separately (profiles/r01g_tmem_cpa.txt, r02_knobs_ab.txt). The row loop is unrolled
+// by a multiple of the window period 3 (TbGeom::UNR) so the W[t][*] rotation is register
+// renaming instead of ~50 moves per row.
 constexpr int kTbCpa = TEA_TB_CPA, kTbCpaL = TEA_TB_CPA_L;
 static_assert(kTbCpa >= 1 && kTbCpaL >= 1 && kTbCpaL <= kTbCpa, "staging depth");
 
@@ -861,8 +854,6 @@ static void tb_dispatch(const KArgs &a, const Region &R, const Region &Dd, int t
     }
 #undef TB
 }
-
-int tb_max_steps() { return 5; }
 
 // Rows per CTA tile: a CTA costs ~ (ty + 2 NL) row-iterations (pipeline fill/drain); an SM
 // holding n CTAs of a wave runs them at a rate that grows with n but saturates (the passes
