@@ -145,21 +145,13 @@ __device__ __forceinline__ void tm_st16(uint32_t a, double2 v0, double2 v1, doub
         "r"(d_hi(v3.y))
         : "memory");
 }
-__device__ __forceinline__ void tm_st12(uint32_t a, double2 v0, double2 v1, double2 v2) {
-    asm volatile(
-        "tcgen05.st.sync.aligned.32x32b.x8.b32 [%0], {%1, %2, %3, %4, %5, %6, %7, %8};\n\t"
-        "tcgen05.st.sync.aligned.32x32b.x4.b32 [%9], {%10, %11, %12, %13};" ::"r"(a),
-        "r"(d_lo(v0.x)), "r"(d_hi(v0.x)), "r"(d_lo(v0.y)), "r"(d_hi(v0.y)), "r"(d_lo(v1.x)),
-        "r"(d_hi(v1.x)), "r"(d_lo(v1.y)), "r"(d_hi(v1.y)), "r"(a + 8u), "r"(d_lo(v2.x)),
-        "r"(d_hi(v2.x)), "r"(d_lo(v2.y)), "r"(d_hi(v2.y))
-        : "memory");
-}
 #ifndef TEA_TB_STX2
 #define TEA_TB_STX2 1
 #endif
 // One double (an aligned register pair) into two TMEM columns: storing a row slot double by
 // double needs no operand marshalling (the x8 / x4 forms want 8 / 4 consecutive registers:
-// 16 register moves per row, profiles/r02c_ncu_summary.md)
+// 16 register moves per row; with the warp-uniform base: 150.7/151.9 -> 148.8/149.8 us,
+// profiles/r02_stx_ab.txt)
 __device__ __forceinline__ void tm_st1(uint32_t a, double v) {
     asm volatile("tcgen05.st.sync.aligned.32x32b.x2.b32 [%0], {%1, %2};" ::"r"(a), "r"(d_lo(v)),
                  "r"(d_hi(v))
@@ -169,11 +161,22 @@ __device__ __forceinline__ void tm_st2x(uint32_t a, double2 v) {
     tm_st1(a, v.x);
     tm_st1(a + 2u, v.y);
 }
+#if !TEA_TB_STX2  // round 1: a row slot as one x8 + one x4 store, the diagonal as x4
+__device__ __forceinline__ void tm_st12(uint32_t a, double2 v0, double2 v1, double2 v2) {
+    asm volatile(
+        "tcgen05.st.sync.aligned.32x32b.x8.b32 [%0], {%1, %2, %3, %4, %5, %6, %7, %8};\n\t"
+        "tcgen05.st.sync.aligned.32x32b.x4.b32 [%9], {%10, %11, %12, %13};" ::"r"(a),
+        "r"(d_lo(v0.x)), "r"(d_hi(v0.x)), "r"(d_lo(v0.y)), "r"(d_hi(v0.y)), "r"(d_lo(v1.x)),
+        "r"(d_hi(v1.x)), "r"(d_lo(v1.y)), "r"(d_hi(v1.y)), "r"(a + 8u), "r"(d_lo(v2.x)),
+        "r"(d_hi(v2.x)), "r"(d_lo(v2.y)), "r"(d_hi(v2.y))
+        : "memory");
+}
 __device__ __forceinline__ void tm_st4(uint32_t a, double2 v) {
     asm volatile("tcgen05.st.sync.aligned.32x32b.x4.b32 [%0], {%1, %2, %3, %4};" ::"r"(a),
                  "r"(d_lo(v.x)), "r"(d_hi(v.x)), "r"(d_lo(v.y)), "r"(d_hi(v.y))
                  : "memory");
 }
+#endif
 struct TmRow {
     uint32_t v[16];
 };
