@@ -572,6 +572,10 @@ def test_compute_sanitizer(tea, tool):
     import shutil
     import subprocess
     import sys
+    # opt-in: the GPU pool closed compute-sanitizer in round 2 (runs under it had left GPUs
+    # needing a reset); the committed reports are under profiles/sanitizers/
+    if os.environ.get("TEA_RUN_SANITIZER") != "1":
+        pytest.skip("compute-sanitizer runs are opt-in (TEA_RUN_SANITIZER=1)")
     exe = shutil.which("compute-sanitizer") or "/usr/local/cuda/bin/compute-sanitizer"
     if not os.path.exists(exe):
         pytest.skip("compute-sanitizer not found")
@@ -579,6 +583,8 @@ def test_compute_sanitizer(tea, tool):
     out = subprocess.run([exe, "--tool", tool, "--error-exitcode", "9", sys.executable,
                           os.path.join(root, "tools", "sanitize.py")], capture_output=True,
                          text=True, timeout=900, cwd=root)
+    if "closed on this pool" in out.stdout + out.stderr:
+        pytest.skip("compute-sanitizer is closed on this GPU pool")
     assert out.returncode == 0, out.stdout[-3000:] + out.stderr[-3000:]
     assert "0 errors" in out.stdout or "0 hazards" in out.stdout
 
