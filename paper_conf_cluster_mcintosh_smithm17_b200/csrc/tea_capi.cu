@@ -455,10 +455,25 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
                 int nrank = nbid / (c->px * c->py / c->nranks);
                 if (nrank != c->rank) remote = true;
             }
-    if (remote) NK(ncclGroupStart());
     const int bpr = c->px * c->py / c->nranks;
     const ncclComm_t hcomm = (xs && c->xcomm) ? c->xcomm : c->comm;
-    for (auto &b : c->blocks) {
+    // NCCL matches the sends and receives between two ranks in posting order: with several
+    // blocks per rank one pair of ranks can carry several messages, so both sides post them
+    // in one canonical order -- (sending block, receiving block, direction seen from the
+    // sender), global block ids
+    struct Msg {
+        int src, dst, dir;
+        double *buf;
+        size_t len;
+        int peer;
+        bool operator<(const Msg &o) const {
+            return src != o.src ? src < o.src : (dst != o.dst ? dst < o.dst : dir < o.dir);
+        }
+    };
+    std::vector<Msg> sends, recvs;
+    for (size_t i = 0; i < c->blocks.size(); ++i) {
+        auto &b = c->blocks[i];
+        const int gid = c->rank * bpr + (int)i;
         const XPlan &x = b.xp[kind];
         for (int d = 0; d < kNDir; ++d) {
             int nbid = b.nbr[d];
@@ -474,14 +489,19 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
                                    x.slen[d] * sizeof(double), cudaMemcpyDeviceToDevice,
                                    st));
             } else {
-                NK(ncclSend(b.sendbuf + x.soff[d], x.slen[d], ncclDouble, nrank, hcomm,
-                            st));
-                NK(ncclRecv(b.recvbuf + x.roff[d], x.rlen[d], ncclDouble, nrank, hcomm,
-                            st));
+                sends.push_back({gid, nbid, d, b.sendbuf + x.soff[d], x.slen[d], nrank});
+                recvs.push_back({nbid, gid, kOpp[d], b.recvbuf + x.roff[d], x.rlen[d], nrank});
             }
         }
     }
-    if (remote) NK(ncclGroupEnd());
+    if (remote) {
+        std::sort(sends.begin(), sends.end());
+        std::sort(recvs.begin(), recvs.end());
+        NK(ncclGroupStart());
+        for (const Msg &m : sends) NK(ncclSend(m.buf, m.len, ncclDouble, m.peer, hcomm, st));
+        for (const Msg &m : recvs) NK(ncclRecv(m.buf, m.len, ncclDouble, m.peer, hcomm, st));
+        NK(ncclGroupEnd());
+    }
     for (auto &b : c->blocks) {
         const XPlan &x = b.xp[kind];
         if (x.nrecv == 0) continue;

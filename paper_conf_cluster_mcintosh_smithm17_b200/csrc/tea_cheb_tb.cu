@@ -323,6 +323,9 @@ struct TbGeom {
     static constexpr int UNR = D == 6 ? 6 : 3;
 };
 
+#ifndef TEA_TB_FILL
+#define TEA_TB_FILL 1  // skip the cone-exterior level-rows of the pipeline fill
+#endif
 #ifndef TEA_TB_MINB
 #define TEA_TB_MINB 3
 #endif
@@ -510,8 +513,13 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                           // pipeline-fill rows every pass discards)
     const double hrx = a.hrx, hry = a.hry;
     constexpr int UNR = G::UNR;
-#pragma unroll(UNR)
-    for (int k = kbeg; k < kend; ++k, orow += pitch, head = head + 1 == D ? 0 : head + 1) {
+    // One row-iteration: input row k, level t on row k - t. fi = k - kbeg during the pipeline
+    // fill (TEA_TB_FILL), else large: level t's rows below kt0 - (NL - t) are outside the
+    // tile's cone (no later level reads them) and are first needed at fi = 2t, so the first
+    // 2 NL row-iterations skip their arithmetic -- NL (NL + 1) of the (ty + 2 NL) NL level-rows
+    // a tile computed (30 of 985 at ty = 187; 30 of 240 on the ~38-row tiles of 2048 x 1024
+    // blocks).
+    auto row = [&](const int k, const int fi) {
         cp_wait<P - 1>();  // row k's group (the oldest outstanding) has landed
         double2 X = cpa[cs][0][threadIdx.x];
         double2 KX, KY;
@@ -621,13 +629,14 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
             // Kx(jA+2) X(jA+2), is the east lane's own Kx(jA) X(jA) -- one product shuffled.
             // Dependency order: xp (the "up" row) is the row level t-1 produced in THIS
             // row-iteration; everything else is older. Form the rest first, fold xp in last.
+            double2 zn = z0;
+            if (fi >= 2 * t) {  // (fill: a compile-time constant per unrolled iteration)
             const double left = __shfl_up_sync(0xffffffffu, xc.y, 1);
             const double east = __shfl_down_sync(0xffffffffu, kx.x * xc.x, 1);
             double2 nb;  // sum_f K_f X_f - d X without the up face (Listing 1)
             nb.x = fma(-dg.x, xc.x, fma(kx.x, left, fma(kx.y, xc.y, kyc.x * xm.x)));
             nb.y = fma(-dg.y, xc.y, fma(kx.y, xc.x, fma(kyc.y, xm.y, east)));
             const bool rowout = q >= kt0 && q < kt1;
-            double2 zn = z0;
             if (PRE && t == 1) {
                 // w = A p; r' = r - alpha w = r + alpha (sum_f K_f p_f - d p)
                 zn.x = fma(alpha, fma(kyn.x, xp.x, nb.x), rq.x);
@@ -709,6 +718,7 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                     }
                 }
             }
+            }  // fi >= 2t
             if (t < NL) {
                 const int tt = t < NL ? t : NL - 1;
                 W[tt][0] = W[tt][1];
@@ -722,7 +732,20 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                 s_d = tm_get(tmB, 3);
             }
         }
-    }
+    };
+    int k = kbeg;
+#if TEA_TB_FILL
+    // the fill, fully unrolled (every fi, slot and window index a constant); a multiple of the
+    // main loop's unroll, so the main loop starts on ring and staging slot 0 as before. A tile
+    // shorter than the fill runs its extra row-iterations on rows past kend: nothing of them
+    // is stored or summed (every store and dot is limited to rows < kt1).
+    constexpr int kFill = (2 * NL + UNR - 1) / UNR * UNR;
+#pragma unroll
+    for (int i = 0; i < kFill; ++i, ++k, orow += pitch, head = head + 1 == D ? 0 : head + 1)
+        row(k, i);
+#endif
+#pragma unroll(UNR)
+    for (; k < kend; ++k, orow += pitch, head = head + 1 == D ? 0 : head + 1) row(k, 1 << 20);
     asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory");
     __syncthreads();
     if ((threadIdx.x >> 5) == 0)

@@ -16,7 +16,7 @@ for p in re.split(r"\n\s+Function : ", txt):
         continue
     ins = []
     for l in p.split("\n"):
-        m = re.search(r"/\*([0-9a-f]{4})\*/\s+(.*?);", l)
+        m = re.search(r"/\*([0-9a-f]{4,6})\*/\s+(.*?);", l)
         if m:
             ins.append((int(m.group(1), 16), m.group(2).strip()))
     back = []
