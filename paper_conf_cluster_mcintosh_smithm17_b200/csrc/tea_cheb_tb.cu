@@ -882,15 +882,22 @@ static void tb_dispatch(const KArgs &a, const Region &R, const Region &Dd, int t
 }
 
 // Rows per CTA tile: a CTA costs ~ (ty + 2 NL) row-iterations (pipeline fill/drain); an SM
-// holding n CTAs of a wave runs them at a rate that grows with n but saturates (the passes
-// are latency-bound with few warps, issue-bound with 3 CTAs), modelled as n / (n + 1/2): a
-// launch costs waves x (ty + 2 NL) x (n + 1/2). This keeps 4096^2's full wave of 187-row
-// tiles and picks fewer, taller tiles where a full wave would make them short (2048 x 1024
-// blocks: 24-row tiles at 3 CTAs per SM 393 / 460 us vs 32-row tiles at ~2.2 per SM 360 /
-// 385 us per 5 timesteps, profiles/r02_blocks_ab.txt). The occupancy is computed from the
+// holding n CTAs of a wave runs them at a rate that saturates at ~2 CTAs (tb_row_time): a
+// launch costs the sum over its waves of (ty + 2 NL) x tb_row_time(CTAs on the busiest SM).
+// This keeps 4096^2's full wave of 187-row tiles, ~36-row tiles at 2 CTAs per SM on 2048 x
+// 1024 blocks (24-row tiles at 3 per SM: 26.8/29.9 vs 25.5/30.2 us) and 18-row tiles at
+// 1024^2 (14.5/17.8 vs 17.5/20.1 us with 25). The occupancy is computed from the
 // kernel's registers and shared memory: cudaOccupancyMaxActiveBlocksPerMultiprocessor reports
 // 1 CTA per SM for these kernels while 3 are resident (ncu), which made every earlier plan a
 // "3-wave" one.
+// Relative row-iteration time of a fused-pass CTA when its SM holds n of them (round 2
+// sweeps, profiles/r02_tbrows_model.txt): ~0.5 us with 2 CTAs per SM and ~0.7 us with 3 at
+// 1965 MHz (1024^2, 2048^2, 2 x 4 blocks of 4096^2): an SM's throughput barely grows past 8
+// warps, so a plan with one CTA less on the busiest SM can win with taller
+// tiles. (Round 2a modelled n / (n + 1/2) on the average count: 25-row tiles at 1024^2, 8%
+// slower than 18.)
+static double tb_row_time(int n) { return n <= 1 ? 0.7 : (n == 2 ? 1.0 : 0.47 * n); }
+
 int tb_auto_rows(int NL, int width, int height) {
     static std::atomic<int> slot_cache[kMaxDev][8];
     static std::atomic<int> sm_cache[kMaxDev];
@@ -939,10 +946,12 @@ int tb_auto_rows(int NL, int width, int height) {
     // per first pass, profiles/r02_blocks_ab.txt)
     for (int ty = std::max(1, height / 4096); ty <= std::min(height, 512); ++ty) {
         const long long ctas = (long long)gx * ((height + ty - 1) / ty);
-        const long long waves = (ctas + slots - 1) / slots;
-        const double per_sm = waves > 1 ? (double)slots / nsm
-                                         : std::max(1.0, (double)(ctas - (waves - 1) * slots) / nsm);
-        const double cost = (double)waves * (ty + 2 * NL) * (per_sm + 0.5);
+        const long long full = ctas / slots, rest = ctas - full * slots;
+        // a wave lasts as long as its busiest SM: (ty + 2 NL) row-iterations at the rate of
+        // the CTA count that SM holds (ceil, not the average)
+        const double cost =
+            (ty + 2 * NL) * ((double)full * tb_row_time(slots / nsm) +
+                             (rest ? tb_row_time((int)((rest + nsm - 1) / nsm)) : 0.0));
         if (cost < bestc - 1e-9) {
             bestc = cost;
             best = ty;
