@@ -210,6 +210,16 @@ __device__ __forceinline__ void tm_wait_ld(TmRow &o) {
                  :
                  : "memory");
 }
+// no use of o's registers moves above this point (after a tm_wait_ld that covered its load)
+__device__ __forceinline__ void tm_pin(TmRow &o) {
+    asm volatile(""
+                 : "+r"(o.v[0]), "+r"(o.v[1]), "+r"(o.v[2]), "+r"(o.v[3]), "+r"(o.v[4]),
+                   "+r"(o.v[5]), "+r"(o.v[6]), "+r"(o.v[7]), "+r"(o.v[8]), "+r"(o.v[9]),
+                   "+r"(o.v[10]), "+r"(o.v[11]), "+r"(o.v[12]), "+r"(o.v[13]), "+r"(o.v[14]),
+                   "+r"(o.v[15])
+                 :
+                 : "memory");
+}
 __device__ __forceinline__ void tm_wait_st() {
     asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
 }
@@ -323,6 +333,12 @@ struct TbGeom {
     static constexpr int UNR = D == 6 ? 6 : 3;
 };
 
+#ifndef TEA_TB_LDPAIR
+#define TEA_TB_LDPAIR 0  // fetch two levels' TMEM slots per round trip in every pass
+#endif
+#ifndef TEA_TB_MINB_PRE
+#define TEA_TB_MINB_PRE 2  // CPPCG1F's 6-level first pass: 2 CTAs/SM, no spills
+#endif
 #ifndef TEA_TB_FILL
 #define TEA_TB_FILL 1  // skip the cone-exterior level-rows of the pipeline fill
 #endif
@@ -348,7 +364,7 @@ constexpr int kTmCols = 128;  // TMEM columns per 4 warps: 8 slots x 16 per warp
 // the update the SpMV otherwise applies lazily, moved to the compute-bound last pass whose HBM
 // bandwidth is idle (SpMV 7 -> 5 streams, this pass 5 -> 8).
 template <int M, bool FIRST, bool FUSE, bool LAST, bool KG, bool PRE, bool POST, bool UPD = false>
-__global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
+__global__ void __launch_bounds__(kTbT, PRE ? TEA_TB_MINB_PRE : TEA_TB_MINB)
     k_cheb_tb(const double *__restrict__ rin, const double *__restrict__ win,
               double *__restrict__ rout, const double *__restrict__ zin1,
               const double *__restrict__ zin2, double *__restrict__ zoutA,
@@ -363,6 +379,9 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
     constexpr bool POSTF = POST && ((M + (PRE ? 1 : 0)) % 2 == 1);
     constexpr int NL = M + (PRE ? 1 : 0) + ((POST && !POSTF) ? 1 : 0);  // stencil levels
     constexpr int T0 = PRE ? 2 : 1;                         // level of the first Chebyshev step
+    // paired TMEM slot fetches: CPPCG1F's last pass 168 -> 160 us at 4096^2, the CPPCG passes
+    // unchanged or slower (profiles/r02_ldpair_ab.txt)
+    constexpr bool kPair = TEA_TB_LDPAIR || POST;
     using G = TbGeom<NL>;
     constexpr int D = G::D;
     static_assert(NL <= 6, "the TMEM ring holds NL+2 rows");
@@ -613,12 +632,23 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
         W[0][0] = W[0][1];
         W[0][1] = W[0][2];
         W[0][2] = X;
+        TmRow tmC;  // kPair: the even level's slot, fetched with the odd level's
+        (void)tmC;
 #pragma unroll
         for (int t = 1; t <= NL; ++t) {
             const int q = k - t;
             // issue the next level's slot (row q-1) before computing this one
             TmRow tmB;
+            if constexpr (kPair) {
+            // odd levels fetch the next TWO levels' slots in one round trip (3 per row
+            // instead of 5 at NL = 5); the second waits in tmC for the even level
+            if (t < NL && t % 2 == 1) {
+                tm_ld16(tm + 16u * ((head + 2 * D - t - 1) % D), tmB);
+                if (t + 1 < NL) tm_ld16(tm + 16u * ((head + 2 * D - t - 2) % D), tmC);
+            }
+            } else {
             if (t < NL) tm_ld16(tm + 16u * ((head + 2 * D - t - 1) % D), tmB);
+            }
             const double2 kx = s_kx, kyc = s_ky, rq = s_r;
             const double2 xm = W[t - 1][0], xc = W[t - 1][1], xp = W[t - 1][2];
             const double2 dg = s_d;
@@ -724,12 +754,28 @@ __global__ void __launch_bounds__(kTbT, TEA_TB_MINB)
                 W[tt][0] = W[tt][1];
                 W[tt][1] = W[tt][2];
                 W[tt][2] = zn;
-                tm_wait_ld(tmB);
                 kyn = kyc;  // Ky of row q = the top faces of row q-1
+                if constexpr (kPair) {
+                if (t % 2 == 1) {
+                    tm_wait_ld(tmB);
+                    if (t + 1 < NL) tm_pin(tmC);
+                    s_kx = tm_get(tmB, 0);
+                    s_ky = tm_get(tmB, 1);
+                    s_r = tm_get(tmB, 2);
+                    s_d = tm_get(tmB, 3);
+                } else {
+                    s_kx = tm_get(tmC, 0);
+                    s_ky = tm_get(tmC, 1);
+                    s_r = tm_get(tmC, 2);
+                    s_d = tm_get(tmC, 3);
+                }
+                } else {
+                tm_wait_ld(tmB);
                 s_kx = tm_get(tmB, 0);
                 s_ky = tm_get(tmB, 1);
                 s_r = tm_get(tmB, 2);
                 s_d = tm_get(tmB, 3);
+                }
             }
         }
     };
@@ -919,7 +965,10 @@ int tb_auto_rows(int NL, int width, int height) {
     case (m + (POST ? 1 : 0)):                                                                   \
         e = cudaFuncGetAttributes(&fa, k_cheb_tb<m, false, false, true, true, false, POST>);     \
         break;
-            OCC(1, false) OCC(2, false) OCC(3, false) OCC(4, false) OCC(5, false) OCC(5, true)
+            OCC(1, false) OCC(2, false) OCC(3, false) OCC(4, false) OCC(5, false)
+            case 6:  // CPPCG1F's first pass (PRE + 5 steps), compiled for 2 CTAs/SM
+                e = cudaFuncGetAttributes(&fa, k_cheb_tb<5, true, false, false, true, true, false>);
+                break;
 #undef OCC
         }
         if (e == cudaSuccess && fa.numRegs > 0) {
