@@ -40,8 +40,10 @@ namespace tea {
 constexpr int kTbW = TEA_TB_WARPS;
 constexpr int kTbT = 32 * kTbW;
 #ifndef TEA_TB_CPA
-#define TEA_TB_CPA 6  // rows of cp.async input staging ahead of the march (first pass): 4 -> 6
-                      // rows, 184 -> 164 us at 4096^2 (profiles/r02_knobs_ab.txt)
+#define TEA_TB_CPA 5  // rows of cp.async input staging ahead of the march (first pass): 4 -> 6
+                      // rows, 184 -> 164 us at 4096^2 (profiles/r02_knobs_ab.txt); 6 -> 5: the
+                      // 6 staging slots cycle with the 6-row unroll (compile-time slot indices,
+                      // 48 fewer instructions per 6 rows; profiles/r02_cpa_ab.txt)
 #endif
 constexpr int kTbNS = 5;  // staged streams per row (X, W or z_{i-2}, r, Kx, Ky)
 
@@ -287,7 +289,8 @@ __device__ bool grid_arrive2(unsigned *ticket) {
 }  // namespace
 
 #ifndef TEA_TB_CPA_L
-#define TEA_TB_CPA_L 2
+#define TEA_TB_CPA_L 5  // later passes: 2 -> 5 rows (ncu: 11% of the last pass's stall samples on
+                        // the staged-row LDS waiting for its cp.async; 147.7 -> 146.0 us)
 #endif
 // cp.async depth of the first pass (carries r, w and the update) and of the later passes,
 // measured separately (profiles/r01g_tmem_cpa.txt, r02_knobs_ab.txt). The row loop is unrolled
@@ -298,9 +301,16 @@ static_assert(kTbCpa >= 1 && kTbCpaL >= 1 && kTbCpaL <= kTbCpa, "staging depth")
 
 // dynamic shared memory of a pass: the cp.async row staging; at least 48 KB so at most 4
 // CTAs are resident per SM and 4 x kTmCols TMEM columns always fit in the SM's 512
+// staged (stream, row) slots of a pass: kTbNS streams (6 with UPD's p and u in a later pass)
+// x (staging depth + 1) rows
+template <bool FIRST, bool UPD>
+__host__ __device__ constexpr int tb_slot_rows() {
+    return ((UPD && !FIRST) ? 6 : kTbNS) * ((FIRST ? kTbCpa : kTbCpaL) + 1);
+}
+template <bool FIRST, bool UPD>
 constexpr size_t tb_smem_bytes() {
-    return sizeof(double2) * kTbNS * (kTbCpa + 1) * kTbT > 48u * 1024u
-               ? sizeof(double2) * kTbNS * (kTbCpa + 1) * kTbT
+    return sizeof(double2) * tb_slot_rows<FIRST, UPD>() * kTbT > 48u * 1024u
+               ? sizeof(double2) * tb_slot_rows<FIRST, UPD>() * kTbT
                : 48u * 1024u;
 }
 
@@ -489,7 +499,7 @@ __global__ void __launch_bounds__(kTbT, PRE ? TEA_TB_MINB_PRE : TEA_TB_MINB)
     // warp. With one register-prefetched row the pass stalled on the load of the next row
     // (ncu: 41% of stall samples on its first use; profiles/r01g_tmem_cpa.txt).
     constexpr int P = FIRST ? kTbCpa : kTbCpaL, NSL = P + 1;
-    static_assert(NS * NSL <= kTbNS * (kTbCpa + 1), "staging fits the dynamic shared memory");
+    static_assert(NS * NSL <= tb_slot_rows<FIRST, UPD>(), "staging fits the dynamic shared memory");
     double2(*cpa)[NS][kTbT] = reinterpret_cast<double2(*)[NS][kTbT]>(tb_smem);
     for (int sl = 0; sl < NSL; ++sl)
 #pragma unroll
@@ -856,7 +866,7 @@ static void tb_launch(const KArgs &a, const Region &R, const Region &Dd, int ty,
     const int width = R.j1 - (R.j0 & (TEA_TB_GEOM == 2 ? ~3 : ~1));
     const int ow = tb_out_cols(NL);
     dim3 grid((width + ow - 1) / ow, (R.k1 - R.k0 + ty - 1) / ty);
-    constexpr size_t smem = tb_smem_bytes();
+    constexpr size_t smem = tb_smem_bytes<FIRST, UPD>();
     // > 48 KB of dynamic shared memory needs the attribute, set once per device
     static std::atomic<unsigned long long> attr{0ull};  // per instantiation: device bit mask
     const unsigned long long bit = 1ull << tea_device();
@@ -954,7 +964,8 @@ int tb_auto_rows(int NL, int width, int height) {
         int nsm = 148, per = 0, smem_sm = 0;
         cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, dev);
         cudaDeviceGetAttribute(&smem_sm, cudaDevAttrMaxSharedMemoryPerMultiprocessor, dev);
-        const size_t smem = tb_smem_bytes();
+        // (the larger of the first and later passes' staging: one plan serves both)
+        const size_t smem = std::max(tb_smem_bytes<true, false>(), tb_smem_bytes<false, false>());
         cudaError_t e = cudaSuccess;
         // resident CTAs per SM from the kernel's registers and shared memory (the occupancy
         // API reports 1 for these kernels, round 2 probe -- ncu shows ~3 resident), capped
