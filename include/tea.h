@@ -273,6 +273,17 @@ tea_status tea_block_extent(const tea_mesh *mesh, int px, int py, int b, int *x0
  * A block without neighbours uses the same schedule with every exchange a no-op. */
 int tea_cheb_schedule(int s, int d, int *ops, int cap);
 
+/* Cross-process halo messages of `rank` for one exchange at halo depth `depth` (corners
+ * when `corners` != 0, `nfields` fields per box), in the order tea_solve posts them inside
+ * one NCCL group: all sends, then all receives, each sorted by (sending block, receiving
+ * block, direction from the sender) -- the canonical order both ranks of a pair share (NCCL
+ * matches a pair's point-to-point calls in posting order). Writes up to cap
+ * 6-tuples (op 0 send / 1 recv, peer rank, sending block, receiving block, direction
+ * 0..7 = W, E, S, N, SW, SE, NW, NE, length in doubles) into out[6*i..6*i+5] and returns
+ * the message count (when it exceeds cap nothing is written), or a negative tea_status. */
+int tea_halo_order(const tea_mesh *mesh, int px, int py, int nranks, int rank, int depth,
+                   int corners, int nfields, long long *out, int cap);
+
 #ifdef __cplusplus
 }
 #endif

@@ -29,7 +29,7 @@ KERNELS = ["init", "residual", "spmv", "update", "cheb_first", "cheb_step", "che
 SYMBOLS = ["tea_version", "tea_abi_version", "tea_get_nccl_id", "tea_workspace_bytes", "tea_init",
            "tea_solve", "tea_fetch", "tea_set_u", "tea_kernel_times", "tea_launch_count",
            "tea_finalize", "tea_last_error", "tea_block_extent", "tea_cheb_schedule",
-           "tea_trace_read"]
+           "tea_halo_order", "tea_trace_read"]
 
 
 class TeaError(RuntimeError):
@@ -108,6 +108,7 @@ def lib(build_if_needed: bool = True):
     L.tea_last_error.restype = C.c_char_p
     L.tea_block_extent.argtypes = [C.POINTER(Mesh), i, i, i] + [C.POINTER(C.c_int)] * 4
     L.tea_cheb_schedule.argtypes = [i, i, vp, i]
+    L.tea_halo_order.argtypes = [C.POINTER(Mesh), i, i, i, i, i, i, i, vp, i]
     L.tea_trace_read.argtypes = [vp, i, vp, vp, vp, vp, i]
     _lib = L
     return L
@@ -159,6 +160,20 @@ def cheb_schedule(s: int, d: int):
     if n < 0:
         raise TeaError(n, "bad schedule arguments")
     return [(buf[2 * i], buf[2 * i + 1]) for i in range(n)]
+
+
+def halo_order(mesh: Mesh, px: int, py: int, nranks: int, rank: int, depth: int,
+               corners: bool = True, nfields: int = 1):
+    """Cross-process halo messages of `rank` in the order tea_solve posts them (host-only):
+    [(op 0 send / 1 recv, peer, sending block, receiving block, direction, length)]."""
+    n = lib().tea_halo_order(C.byref(mesh), px, py, nranks, rank, depth, int(corners), nfields,
+                             None, 0)
+    if n < 0:
+        raise TeaError(n, "bad halo_order arguments")
+    buf = (C.c_longlong * (6 * max(n, 1)))()
+    lib().tea_halo_order(C.byref(mesh), px, py, nranks, rank, depth, int(corners), nfields,
+                         buf, n)
+    return [tuple(buf[6 * k:6 * k + 6]) for k in range(n)]
 
 
 def _f64(a):

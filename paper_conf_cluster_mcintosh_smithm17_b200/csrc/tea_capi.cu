@@ -413,6 +413,27 @@ void reduce(tea_ctx *c, int first, int n) {
 }
 
 // ------------------------------------------------------------------ halo exchange
+// One cross-process halo message: global ids of the sending and receiving block, the
+// direction seen from the sender, its length (doubles), the peer rank and the local buffer.
+struct HaloMsg {
+    int src, dst, dir;
+    double *buf;
+    size_t len;
+    int peer;
+    bool operator<(const HaloMsg &o) const {
+        return src != o.src ? src < o.src : (dst != o.dst ? dst < o.dst : dir < o.dir);
+    }
+};
+// NCCL matches the sends and receives between two ranks in posting order: with several
+// blocks per rank one pair of ranks can carry several messages (a face and a corner to two
+// blocks of the same rank, possibly of equal size), so both sides post them in ONE canonical
+// order -- (sending block, receiving block, direction seen from the sender). Shared by the
+// exchange and the host-only tea_halo_order (tests/test_dist_gloo.py replays it over gloo).
+void halo_post_order(std::vector<HaloMsg> &sends, std::vector<HaloMsg> &recvs) {
+    std::sort(sends.begin(), sends.end());
+    std::sort(recvs.begin(), recvs.end());
+}
+
 void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field,
               cudaStream_t xs = nullptr) {
     // fids: field ids (same for every block), 1 or 2 entries; xs: the stream to run on
@@ -457,20 +478,7 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
             }
     const int bpr = c->px * c->py / c->nranks;
     const ncclComm_t hcomm = (xs && c->xcomm) ? c->xcomm : c->comm;
-    // NCCL matches the sends and receives between two ranks in posting order: with several
-    // blocks per rank one pair of ranks can carry several messages, so both sides post them
-    // in one canonical order -- (sending block, receiving block, direction seen from the
-    // sender), global block ids
-    struct Msg {
-        int src, dst, dir;
-        double *buf;
-        size_t len;
-        int peer;
-        bool operator<(const Msg &o) const {
-            return src != o.src ? src < o.src : (dst != o.dst ? dst < o.dst : dir < o.dir);
-        }
-    };
-    std::vector<Msg> sends, recvs;
+    std::vector<HaloMsg> sends, recvs;
     for (size_t i = 0; i < c->blocks.size(); ++i) {
         auto &b = c->blocks[i];
         const int gid = c->rank * bpr + (int)i;
@@ -495,11 +503,10 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
         }
     }
     if (remote) {
-        std::sort(sends.begin(), sends.end());
-        std::sort(recvs.begin(), recvs.end());
+        halo_post_order(sends, recvs);
         NK(ncclGroupStart());
-        for (const Msg &m : sends) NK(ncclSend(m.buf, m.len, ncclDouble, m.peer, hcomm, st));
-        for (const Msg &m : recvs) NK(ncclRecv(m.buf, m.len, ncclDouble, m.peer, hcomm, st));
+        for (const HaloMsg &m : sends) NK(ncclSend(m.buf, m.len, ncclDouble, m.peer, hcomm, st));
+        for (const HaloMsg &m : recvs) NK(ncclRecv(m.buf, m.len, ncclDouble, m.peer, hcomm, st));
         NK(ncclGroupEnd());
     }
     for (auto &b : c->blocks) {
@@ -1972,6 +1979,48 @@ tea_status tea_block_extent(const tea_mesh *mesh, int px, int py, int b, int *x0
     split(mesh->nx, px, b % px, x0, x1);
     split(mesh->ny, py, b / px, y0, y1);
     return TEA_OK;
+}
+
+int tea_halo_order(const tea_mesh *mesh, int px, int py, int nranks, int rank, int depth,
+                   int corners, int nfields, long long *out, int cap) {
+    if (!mesh || px < 1 || py < 1 || nranks < 1 || (px * py) % nranks || rank < 0 ||
+        rank >= nranks || depth < 1 || nfields < 1 || (!out && cap > 0))
+        return TEA_ERR_ARG;
+    const int bpr = px * py / nranks;
+    std::vector<HaloMsg> sends, recvs;
+    for (int i = 0; i < bpr; ++i) {
+        const int gid = rank * bpr + i, bi = gid % px, bj = gid / px;
+        int x0, x1, y0, y1;
+        split(mesh->nx, px, bi, &x0, &x1);
+        split(mesh->ny, py, bj, &y0, &y1);
+        const int bx = x1 - x0, by = y1 - y0;
+        for (int d = 0; d < kNDir; ++d) {
+            const int ni = bi + kDX[d], nj = bj + kDY[d];
+            if (ni < 0 || ni >= px || nj < 0 || nj >= py) continue;
+            if (d >= 4 && !corners) continue;
+            const int nbid = nj * px + ni, nrank = nbid / bpr;
+            if (nrank == rank) continue;
+            // the send box of build_xplans (send_box): depth columns / rows / both
+            const size_t len = (size_t)nfields * (kDX[d] ? depth : bx) * (kDY[d] ? depth : by);
+            sends.push_back({gid, nbid, d, nullptr, len, nrank});
+            recvs.push_back({nbid, gid, kOpp[d], nullptr, len, nrank});
+        }
+    }
+    halo_post_order(sends, recvs);
+    const int n = (int)(sends.size() + recvs.size());
+    if (n > cap) return n;  // the count only
+    int k = 0;
+    for (int op = 0; op < 2; ++op)
+        for (const HaloMsg &m : op ? recvs : sends) {
+            long long *o = out + 6 * k++;
+            o[0] = op;
+            o[1] = m.peer;
+            o[2] = m.src;
+            o[3] = m.dst;
+            o[4] = m.dir;
+            o[5] = (long long)m.len;
+        }
+    return n;
 }
 
 int tea_cheb_schedule(int s, int d, int *ops, int cap) {

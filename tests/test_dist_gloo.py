@@ -265,3 +265,110 @@ def test_nccl_id_broadcast_over_process_group():
     for p in procs:
         p.join(timeout=60)
     assert len(got[0]) == 128 and got[0] == got[1] and any(got[0])
+
+
+# ---------------------------------------------------------------- halo message order
+# NCCL (like gloo) matches the point-to-point calls between two ranks in posting order. With
+# several blocks per rank a rank pair carries several messages, some of equal size; the
+# library posts them in one canonical order (tea_halo_order). Each rank replays the LIBRARY's
+# order over gloo isend/irecv (one tag, FIFO per pair) with payloads that name the message;
+# every receive must get exactly the message it was posted for.
+HALO_CASES = [  # (nx, ny, px, py, nranks, depth, corners)
+    (64, 48, 2, 2, 2, 3, True),    # a face and an equal-sized corner cross between 2 ranks
+    (64, 48, 4, 2, 2, 4, True),
+    (96, 64, 2, 4, 4, 11, True),
+    (90, 60, 3, 2, 2, 2, True),    # 3 blocks per rank, ragged extents
+    (80, 80, 4, 4, 2, 1, False),   # depth 1, faces only
+    (80, 80, 4, 4, 4, 5, True),
+]
+
+
+def _code(src, dst, d):
+    return float((src * 64 + dst) * 8 + d)
+
+
+def _halo_worker(rank, world, port, cases, q):
+    import torch
+    import torch.distributed as dist
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    sys.path.insert(0, ROOT)
+    import paper_conf_cluster_mcintosh_smithm17_b200 as tea
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    res = []
+    for (nx, ny, px, py, nranks, depth, corners) in cases:
+        if nranks != world:
+            continue
+        msgs = tea.halo_order(tea.make_mesh(nx, ny), px, py, nranks, rank, depth, corners)
+        reqs, recv = [], []
+        for op, peer, src, dst, d, n in msgs:
+            if op == 0:
+                t = torch.full((n,), _code(src, dst, d), dtype=torch.float64)
+                reqs.append(dist.isend(t, int(peer), tag=7))
+        for op, peer, src, dst, d, n in msgs:
+            if op == 1:
+                t = torch.zeros(n, dtype=torch.float64)
+                reqs.append(dist.irecv(t, int(peer), tag=7))
+                recv.append((src, dst, d, t))
+        for r in reqs:
+            r.wait()
+        ok = all(bool(torch.all(t == _code(s, dd, d))) for s, dd, d, t in recv)
+        res.append(((nx, ny, px, py, nranks, depth, corners), ok, len(msgs)))
+    dist.barrier()
+    dist.destroy_process_group()
+    q.put((rank, res))
+
+
+@pytest.mark.parametrize("world", [2, 4])
+def test_halo_message_order_over_gloo(world):
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = free_port()
+    procs = [ctx.Process(target=_halo_worker, args=(r, world, port, HALO_CASES, q))
+             for r in range(world)]
+    for p in procs:
+        p.start()
+    got = dict(q.get(timeout=180) for _ in range(world))
+    for p in procs:
+        p.join(timeout=60)
+    for r in range(world):
+        assert got[r], "no case ran"
+        for case, ok, n in got[r]:
+            assert n > 0 and ok, (r, case)
+
+
+def test_halo_message_order_pairs_agree():
+    """Host-only: for every rank pair, A's sends to B equal B's receives from A, in order and
+    length -- and the per-rank block x direction order of round 1 would cross-match the 2 x 2
+    grid on 2 ranks (a corner received into a face's buffer of the same size)."""
+    sys.path.insert(0, ROOT)
+    import paper_conf_cluster_mcintosh_smithm17_b200 as tea
+    for (nx, ny, px, py, nranks, depth, corners) in HALO_CASES:
+        m = tea.make_mesh(nx, ny)
+        per = {r: tea.halo_order(m, px, py, nranks, r, depth, corners) for r in range(nranks)}
+        for a in range(nranks):
+            for b in range(nranks):
+                if a == b:
+                    continue
+                s = [(src, dst, d, n) for op, p, src, dst, d, n in per[a] if op == 0 and p == b]
+                r = [(src, dst, d, n) for op, p, src, dst, d, n in per[b] if op == 1 and p == a]
+                assert s == r, (nx, ny, px, py, nranks, a, b)
+    # round 1: each rank posted (block, direction) pairs in its own loop order
+    m = tea.make_mesh(64, 48)
+    DXY = list(zip(DX, DY))
+
+    def natural(rank, op):
+        out = []
+        for i in range(2):
+            g = rank * 2 + i
+            bi, bj = g % 2, g // 2
+            for d, (dx, dy) in enumerate(DXY):
+                ni, nj = bi + dx, bj + dy
+                if 0 <= ni < 2 and 0 <= nj < 2 and (nj * 2 + ni) // 2 != rank:
+                    nb = nj * 2 + ni
+                    out.append((g, nb, d) if op == 0 else (nb, g, [1, 0, 3, 2, 7, 6, 5, 4][d]))
+        return out
+    assert natural(0, 0) != natural(1, 1)  # the crossing the canonical order removes
+    canon = [(s, t, d) for op, p, s, t, d, n in tea.halo_order(m, 2, 2, 2, 0, 3, True) if op == 0]
+    assert canon == [(s, t, d) for op, p, s, t, d, n in tea.halo_order(m, 2, 2, 2, 1, 3, True)
+                     if op == 1]
