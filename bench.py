@@ -22,7 +22,7 @@ roofline    the dominant kernel = the kernel class with the largest share of the
             its recorded source hash matches the built library's sources.
 cpu_baseline the CPU oracle (oracle/, serial C, 1 thread) timed on bounded
             samples of the same timestep (30 presteps; + the restart and 1 outer
-            iteration; + 1 more outer iteration), its per-phase costs weighted by
+            iteration; + 2 more outer iterations), its per-phase costs weighted by
             the GPU run's own iteration mix (like for like), and matvecs/s.
 
 Usage: python bench.py [--gpus N] [--steps K] [--warmup W] [--impl reference]
@@ -183,7 +183,7 @@ HEADLINE_MIX = (30.0, 253.1)
 
 def oracle_phase_costs(args, deck):
     """Serial oracle costs of the phases of one timestep, measured on bounded samples:
-    two-phase methods run 30 presteps, then 30 + restart + 1 outer, then + 1 more outer
+    two-phase methods run 30 presteps, then 30 + restart + 1 outer, then + 2 more outer
     (t_pre per prestep, t_restart = eigen-estimate + restart chain, t_outer per outer);
     one-phase methods run 20 iterations. Solve time only (faces precomputed)."""
     import oracle
@@ -212,14 +212,16 @@ def oracle_phase_costs(args, deck):
         return time.perf_counter() - t0, r.stats
 
     if args.method in TWO_PHASE:
+        # the per-outer cost from a 2-outer difference: a 1-outer difference of two ~7 s runs
+        # was noise-dominated at 4096^2 (0.44 vs 0.92 s/outer in two runs on one box, round 2)
         t30, s30 = timed(30)
         t31, s31 = timed(31)
-        t32, s32 = timed(32)
-        t_outer = t32 - t31
+        t33, s33 = timed(33)
+        t_outer = (t33 - t31) / 2
         c = {"t_pre": t30 / 30, "t_restart": max(t31 - t30 - t_outer, 0.0), "t_outer": t_outer,
-             "sample_s": t30 + t31 + t32, "matvecs_per_s": (s30["matvecs"] + s31["matvecs"] +
-                                                          s32["matvecs"]) / (t30 + t31 + t32),
-             "sample": "30 presteps; 30 presteps + restart + 1 outer; + 1 more outer"}
+             "sample_s": t30 + t31 + t33, "matvecs_per_s": (s30["matvecs"] + s31["matvecs"] +
+                                                          s33["matvecs"]) / (t30 + t31 + t33),
+             "sample": "30 presteps; 30 presteps + restart + 1 outer; + 2 more outer"}
     else:
         t20, s20 = timed(20)
         c = {"t_it": t20 / 20, "sample_s": t20, "matvecs_per_s": s20["matvecs"] / t20,
