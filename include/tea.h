@@ -96,10 +96,13 @@ typedef struct {
 
 /* Decomposition: px x py blocks, block b = by*px + bx owns the
  * columns/rows given by an even split with the remainder on low-index blocks.
- * The blocks are shared evenly by `nranks` processes (one process per GPU):
- * rank r owns blocks [r*B, (r+1)*B), B = px*py/nranks. nranks == 1 with
- * px*py > 1 runs every block in this process on one GPU (halo transport by
- * device copies instead of NCCL -- same pack/unpack kernels).
+ * The blocks are shared by `nranks` processes (one process per GPU): rank r
+ * owns blocks [r*B, (r+1)*B), B = px*py/nranks; multi-process runs need B = 1
+ * (TEA_ERR_ARG otherwise). nranks == 1 with px*py > 1 runs every block in this
+ * process on one GPU, halos by an on-device copy kernel; with the environment
+ * variable TEA_NCCL_SELF=1 they go through a 1-rank NCCL communicator instead
+ * (send/recv to self, allreduce, chunked graphs: the multi-process code path on
+ * one GPU, bitwise the same results; a diagnostic).
  * halo_depth d >= 1: matrix-powers depth of the CPPCG inner loop.
  * nccl_id: 128-byte ncclUniqueId from tea_get_nccl_id() on rank 0, broadcast by
  * the caller; NULL when nranks == 1. Pass NULL for `dist` to get 1x1, d = 1.  */

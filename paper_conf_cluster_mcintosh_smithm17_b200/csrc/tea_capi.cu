@@ -153,6 +153,12 @@ struct tea_ctx {
     // exchange there may run concurrently with an allreduce on the compute stream, and two
     // concurrent NCCL operations must not share one communicator's connections
     ncclComm_t xcomm = nullptr;
+    // TEA_NCCL_SELF=1 (diagnostic, one process, several blocks): halos and dot products go
+    // through a 1-rank NCCL communicator -- grouped ncclSend/ncclRecv to self in the canonical
+    // order, ncclAllReduce, the split exchange communicator on the second stream, chunked graphs
+    // and the polled host waits -- the multi-process code path, on one GPU (NCCL refuses two
+    // ranks on one device). Results are bitwise those of the device-copy transport.
+    bool nccl_self = false;
     std::string err;
     bool failed = false;
     long long launches = 0;
@@ -218,7 +224,7 @@ struct TeaError {
 // 600) without completion, or on an NCCL error, the communicator is aborted and the call
 // fails with TEA_ERR_NCCL.
 void wait_stream(tea_ctx *c) {
-    if (c->nranks <= 1 || !c->comm) {
+    if (!c->comm) {
         CK(cudaStreamSynchronize(c->stream));
         return;
     }
@@ -404,7 +410,7 @@ void reduce(tea_ctx *c, int first, int n) {
         for (auto &b : c->blocks) L.push_back(b.S);
         K(c, TEA_K_SCALAR, 0.0, [&] { launch_combine(L.data(), nb, n, first, c->stream); });
     }
-    if (c->nranks > 1) {
+    if (c->nranks > 1 || c->nccl_self) {
         double *p = &c->blocks[0].S->red_pw + first;
         K(c, TEA_K_SCALAR, 0.0,
           [&] { launch_mask_done(c->blocks[0].S, first, n, c->rank != 0, c->stream); });
@@ -474,7 +480,7 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
             if (b.nbr[d] >= 0) {
                 int nbid = b.nbr[d];
                 int nrank = nbid / (c->px * c->py / c->nranks);
-                if (nrank != c->rank) remote = true;
+                if (nrank != c->rank || c->nccl_self) remote = true;
             }
     const int bpr = c->px * c->py / c->nranks;
     const ncclComm_t hcomm = (xs && c->xcomm) ? c->xcomm : c->comm;
@@ -487,7 +493,7 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
             int nbid = b.nbr[d];
             if (nbid < 0) continue;
             int nrank = nbid / bpr;
-            if (nrank == c->rank) {
+            if (nrank == c->rank && !c->nccl_self) {
                 BlockCtx &nbk = c->blocks[nbid - c->rank * bpr];
                 const XPlan &y = nbk.xp[kind];
                 int od = kOpp[d];
@@ -528,7 +534,7 @@ void exchange(tea_ctx *c, int kind, const std::vector<int> &fids_per_block_field
 // allreduce is in flight on the compute stream ("the r halo exchange is issued
 // together with the rr allreduce"); joined before the next iteration.
 void reduce_exchange(tea_ctx *c, int first, int n, int kind, const std::vector<int> &fields) {
-    const bool want = c->opts.overlap > 0 || (c->opts.overlap == 0 && c->nranks > 1);
+    const bool want = c->opts.overlap > 0 || (c->opts.overlap == 0 && (c->nranks > 1 || c->nccl_self));
     if (c->px * c->py > 1 && c->xstream && want && !c->profiling) {
         CK(cudaEventRecord(c->ev_fork, c->stream));
         CK(cudaStreamWaitEvent(c->xstream, c->ev_fork, 0));
@@ -850,7 +856,7 @@ int cheb_chain_tb(tea_ctx *c, int s, bool restart, bool fused, int rin, int rout
     // (M rows / columns around it) are owned cells; the frame of the extended region
     // follows the exchange. The first pass must not be the last (its dot products are one
     // grid reduction); profiling keeps every launch on the compute stream.
-    const bool want = c->opts.overlap > 0 || (c->opts.overlap == 0 && c->nranks > 1);
+    const bool want = c->opts.overlap > 0 || (c->opts.overlap == 0 && (c->nranks > 1 || c->nccl_self));
     const bool ovl = blocks && !x.noexch && c->xstream && want && !c->profiling &&
                      passes.size() > 1;
     if (blocks && !x.noexch) {
@@ -1697,9 +1703,13 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
         if (o.overlap < -1 || o.overlap > 1) fail(TEA_ERR_ARG, "bad overlap");
         if (o.kform < -1 || o.kform > 1) fail(TEA_ERR_ARG, "bad kform");
         if (o.trace < 0 || o.trace > 1) fail(TEA_ERR_ARG, "bad trace");
+        const char *nse = std::getenv("TEA_NCCL_SELF");
+        c->nccl_self = nranks == 1 && px * py > 1 && nse && std::atoi(nse) == 1;
         // NCCL kernels inside a WHILE-conditional graph body are not a supported
         // capture target: multi-process runs use chunked graphs (same kernels).
-        if (nranks > 1 && o.loop_mode == 0) o.loop_mode = 1;
+        const char *nsw = std::getenv("TEA_NCCL_SELF_WHILE");  // diagnostic: keep the WHILE graph
+        if ((nranks > 1 || (c->nccl_self && !(nsw && std::atoi(nsw) == 1))) && o.loop_mode == 0)
+            o.loop_mode = 1;
         c->opts = o;
         // every cell this rank stages (its blocks plus the margin; all of a 3D mesh): a
         // density <= 0 would silently become an insulating internal boundary
@@ -1748,6 +1758,11 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
             std::memcpy(&id, dist->nccl_id, sizeof id);
             NK(ncclCommInitRank(&c->comm, nranks, id, rank));
             if (px * py > 1) NK(ncclCommSplit(c->comm, 0, rank, &c->xcomm, nullptr));
+        } else if (c->nccl_self) {
+            ncclUniqueId id;
+            NK(ncclGetUniqueId(&id));
+            NK(ncclCommInitRank(&c->comm, 1, id, 0));
+            NK(ncclCommSplit(c->comm, 0, 0, &c->xcomm, nullptr));
         }
 
         const int bpr = px * py / nranks;
@@ -1827,7 +1842,8 @@ tea_status tea_init(tea_ctx **out, const tea_mesh *mesh, const double *density,
             CK(cudaMemsetAsync(ws + F_Z0 * L.field_bytes, 0, L.field_bytes, c->stream));
             ws += L.total;
         }
-        if (nranks == 1 && px * py > 1 && bpr <= kXMaxBlocks) build_xcopy(c.get());
+        if (nranks == 1 && px * py > 1 && bpr <= kXMaxBlocks && !c->nccl_self)
+            build_xcopy(c.get());
         CK(cudaStreamSynchronize(c->stream));
         c->coef_slot = tb_slot_acquire();
         *out = c.release();
@@ -1961,8 +1977,11 @@ tea_status tea_finalize(tea_ctx *ctx) {
     if (ctx->ev_join) cudaEventDestroy(ctx->ev_join);
     if (ctx->xstream) cudaStreamDestroy(ctx->xstream);
     if (ctx->hS) cudaFreeHost(ctx->hS);
-    if (ctx->xcomm) ncclCommDestroy(ctx->xcomm);
-    if (ctx->comm) ncclCommDestroy(ctx->comm);
+    // a failed context may hold NCCL operations that were captured but never launched (a
+    // failed graph instantiation) or a peer that is gone: ncclCommDestroy can then wait
+    // forever, so it is aborted instead (TEA_NCCL_SELF_WHILE diagnostic, round 2)
+    if (ctx->xcomm) (ctx->failed ? ncclCommAbort : ncclCommDestroy)(ctx->xcomm);
+    if (ctx->comm) (ctx->failed ? ncclCommAbort : ncclCommDestroy)(ctx->comm);
     if (ctx->stream) cudaStreamDestroy(ctx->stream);
     tb_slot_release(ctx->coef_slot);
     delete ctx;
