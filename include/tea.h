@@ -276,6 +276,12 @@ tea_status tea_block_extent(const tea_mesh *mesh, int px, int py, int b, int *x0
  * A block without neighbours uses the same schedule with every exchange a no-op. */
 int tea_cheb_schedule(int s, int d, int *ops, int cap);
 
+/* Rows per CTA tile the fused Chebyshev passes use for a pass of `levels` stencil levels
+ * (1..6) over width x height cells, given `ctas_per_sm` resident CTAs per SM (the library
+ * derives it from the kernel's registers and shared memory) on `nsm` SMs: the cost model of
+ * DESIGN.md §4.4 (a wave costs its busiest SM's CTA count). Returns the rows, or TEA_ERR_ARG. */
+int tea_tb_plan(int levels, int width, int height, int ctas_per_sm, int nsm);
+
 /* Cross-process halo messages of `rank` for one exchange at halo depth `depth` (corners
  * when `corners` != 0, `nfields` fields per box), in the order tea_solve posts them inside
  * one NCCL group: all sends, then all receives, each sorted by (sending block, receiving

@@ -29,7 +29,7 @@ KERNELS = ["init", "residual", "spmv", "update", "cheb_first", "cheb_step", "che
 SYMBOLS = ["tea_version", "tea_abi_version", "tea_get_nccl_id", "tea_workspace_bytes", "tea_init",
            "tea_solve", "tea_fetch", "tea_set_u", "tea_kernel_times", "tea_launch_count",
            "tea_finalize", "tea_last_error", "tea_block_extent", "tea_cheb_schedule",
-           "tea_halo_order", "tea_trace_read"]
+           "tea_halo_order", "tea_tb_plan", "tea_trace_read"]
 
 
 class TeaError(RuntimeError):
@@ -109,6 +109,7 @@ def lib(build_if_needed: bool = True):
     L.tea_block_extent.argtypes = [C.POINTER(Mesh), i, i, i] + [C.POINTER(C.c_int)] * 4
     L.tea_cheb_schedule.argtypes = [i, i, vp, i]
     L.tea_halo_order.argtypes = [C.POINTER(Mesh), i, i, i, i, i, i, i, vp, i]
+    L.tea_tb_plan.argtypes = [i, i, i, i, i]
     L.tea_trace_read.argtypes = [vp, i, vp, vp, vp, vp, i]
     _lib = L
     return L
@@ -160,6 +161,14 @@ def cheb_schedule(s: int, d: int):
     if n < 0:
         raise TeaError(n, "bad schedule arguments")
     return [(buf[2 * i], buf[2 * i + 1]) for i in range(n)]
+
+
+def tb_plan(levels: int, width: int, height: int, ctas_per_sm: int = 3, nsm: int = 148) -> int:
+    """Rows per tile of a fused Chebyshev pass (the library's cost model, host-only)."""
+    n = lib().tea_tb_plan(levels, width, height, ctas_per_sm, nsm)
+    if n < 0:
+        raise TeaError(n, "bad tb_plan arguments")
+    return n
 
 
 def halo_order(mesh: Mesh, px: int, py: int, nranks: int, rank: int, depth: int,

@@ -2042,6 +2042,12 @@ int tea_halo_order(const tea_mesh *mesh, int px, int py, int nranks, int rank, i
     return n;
 }
 
+int tea_tb_plan(int levels, int width, int height, int ctas_per_sm, int nsm) {
+    if (levels < 1 || levels > 6 || width < 1 || height < 1 || ctas_per_sm < 1 || nsm < 1)
+        return TEA_ERR_ARG;
+    return tb_plan_rows(levels, width, height, ctas_per_sm, nsm);
+}
+
 int tea_cheb_schedule(int s, int d, int *ops, int cap) {
     if (s < 1 || s > kMaxS || d < 1 || d > 16) return TEA_ERR_ARG;
     auto v = cheb_schedule(s, d);

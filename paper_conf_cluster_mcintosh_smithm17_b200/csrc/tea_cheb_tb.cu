@@ -996,7 +996,17 @@ int tb_auto_rows(int NL, int width, int height) {
                     cudaGetErrorString(e), nsm);
         sm_cache[dev].store(nsm);
     }
-    const int nsm = std::max(1, sm_cache[dev].load());
+    return tb_plan_rows(NL, width, height, slots / std::max(1, sm_cache[dev].load()),
+                        std::max(1, sm_cache[dev].load()));
+}
+
+// The cost model alone (host-only; tea_tb_plan exports it for tests): rows per tile for a
+// pass of NL levels over width x height cells with `per` CTAs resident per SM on `nsm` SMs.
+int tb_plan_rows(int NL, int width, int height, int per, int nsm) {
+    NL = NL < 1 ? 1 : (NL > 6 ? 6 : NL);
+    per = std::max(1, per);
+    nsm = std::max(1, nsm);
+    const int slots = per * nsm;
     const int ow = tb_out_cols(NL);
     const int gx = (width + ow - 1) / ow;
     int best = height;

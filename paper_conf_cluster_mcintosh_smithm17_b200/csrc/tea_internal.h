@@ -283,6 +283,7 @@ struct TbArgs {
 int tb_out_cols(int levels);
 int tb_ctas(int levels, int width, int height, int ty);
 int tb_auto_rows(int levels, int width, int height);
+int tb_plan_rows(int levels, int width, int height, int ctas_per_sm, int nsm);
 int tb_slot_acquire();  // -1: none free (the context then uses per-step kernels)
 void tb_slot_release(int slot);
 cudaError_t tb_coef_upload(int slot, const Scalars *S, cudaStream_t st);

@@ -168,3 +168,22 @@ def test_no_cpu_fallback():
                 txt = open(os.path.join(root, f)).read()
                 assert "import oracle" not in txt and "from oracle" not in txt
                 assert "tea_oracle" not in txt
+
+
+def test_fused_pass_tile_plan_matches_measured_optima():
+    """The fused passes' tile-height model (tea_tb_plan, host-only) picks the
+    heights the B200 sweeps measured best (profiles/r02_tbrows_model.txt, r02_tbrows_4096.jsonl):
+    4096^2 187 rows (one wave at 3 CTAs/SM: 2219 it/s vs 2021-2150 for 160-293), 1024^2 18
+    (14.5 / 17.8 us per pass vs 17.5 / 20.1 at 25), the 2 x 4 blocks' first pass on ext(6)
+    (2060 x 1036) ~36 (2 CTAs per SM; 24-row tiles at 3 per SM measured slower), 2048^2 a
+    3-per-SM wave near 50 (60 and 71 measured slower)."""
+    import paper_conf_cluster_mcintosh_smithm17_b200 as tea
+    assert tea.tb_plan(5, 4096, 4096) == 187
+    assert tea.tb_plan(5, 1024, 1024) == 18
+    assert 34 <= tea.tb_plan(5, 2060, 1036) <= 38
+    assert 44 <= tea.tb_plan(5, 2048, 2048) <= 52
+    for lv, w, h in [(1, 64, 3), (6, 16384, 16384), (3, 100, 1), (5, 333, 4097)]:
+        ty = tea.tb_plan(lv, w, h)
+        assert 1 <= ty <= min(h, 512)
+    with pytest.raises(tea.TeaError):
+        tea.tb_plan(0, 10, 10)
